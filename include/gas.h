@@ -1,0 +1,123 @@
+/*
+ * gas.h — C ABI of the B200-native GPU-ArraySort hot path (libgas.so).
+ *
+ * The operation (PAPER.md, cited "P:Lx-y" = line of the paper text):
+ *   Definition 1 (§4): given a batch I of N unsorted arrays
+ *   A_1..A_N of n elements, produce I' where every A'_i is A_i arranged as
+ *   a1 <= a2 <= ... <= an. Arrays are independent,
+ *   the result overwrites the input ("in-place", Abstract
+ *   P:L38-39) and the elements are float32 (§7.2). The paper
+ *   bounds the arrays it designs for at ~4000 elements (spectra peaks,
+ *   P:L170-173), hence gas_max_array_len().
+ *
+ * Ordering (reading C-1): "<=" is IEEE 754-2008 §5.10 totalOrder:
+ *   -NaN(quiet, larger payload first) < -NaN(signaling) < -inf < ... < -0
+ *   < +0 < ... < +inf < +sNaN < +qNaN. The result of each array is a
+ *   permutation of its input BIT PATTERNS (no float arithmetic is applied,
+ *   so no NaN is quieted, no subnormal flushed). The output is unique, so
+ *   every correct implementation is bit-identical (reading C-2).
+ *
+ * Conventions for every entry point:
+ *   - Pointers named d_* are DEVICE memory of the current device, owned by
+ *     the caller; the library never allocates on the device-resident entry
+ *     points (zero workspace) and never calls cudaSetDevice.
+ *   - Work is enqueued on `stream` (0 = legacy default stream) and the call
+ *     returns without a host synchronisation. Argument and launch-
+ *     configuration errors are returned synchronously; faults during
+ *     execution surface at the caller's next synchronisation, as usual in
+ *     CUDA.
+ *   - All counts and element offsets are 64-bit; a batch may hold more than
+ *     2^31 elements (e.g. 10^7 x 1000).
+ *   - Functions are reentrant and thread-safe; concurrent calls on
+ *     overlapping memory are the caller's race.
+ *   - No C++ exceptions cross this boundary.
+ */
+#ifndef GAS_H
+#define GAS_H
+
+#include <stdint.h>
+#include <cuda_runtime_api.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef enum gas_status {
+  GAS_SUCCESS = 0,
+  GAS_ERROR_INVALID_VALUE = 1, /* NULL pointer with work to do; negative count/length;
+                                  pointer not 4-byte aligned; bad offsets (GAS_CHECK=1) */
+  GAS_ERROR_UNSUPPORTED = 2,   /* an array longer than gas_max_array_len() */
+  GAS_ERROR_CUDA = 3           /* a CUDA call failed; raw cudaError_t in gas_last_cuda_error() */
+} gas_status;
+
+/*
+ * Fixed-length batch (Definition 1): array i occupies
+ * d_data[i*array_len .. (i+1)*array_len), i in [0, num_arrays); every array is
+ * sorted ascending in place.
+ *   d_data      device pointer, 4-byte aligned (16-byte aligned with
+ *               array_len % 4 == 0 selects 128-bit vector loads/stores).
+ *   num_arrays  N >= 0. array_len n >= 0. N == 0 or n <= 1: no-op, d_data may be NULL.
+ *   n > gas_max_array_len(): GAS_ERROR_UNSUPPORTED, nothing enqueued.
+ * One kernel launch per call.
+ */
+gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len, cudaStream_t stream);
+
+/*
+ * Variable-length batch (BASELINE.json north_star "variable-length offsets
+ * variant"; reading C-16): array i is d_data[d_offsets[i] ..
+ * d_offsets[i+1]), d_offsets is int64[num_arrays+1] in DEVICE memory,
+ * nondecreasing, d_offsets[0] >= 0. Arrays may be empty, adjacent and at any
+ * 4-byte alignment; no byte outside [d_offsets[0], d_offsets[N]) is touched
+ * and no array's bytes are written by another array's work.
+ *   max_array_len  an upper bound on every length (0 = gas_max_array_len());
+ *                  used to skip size classes that cannot occur. A length above
+ *                  it is undefined behaviour unless the environment variable
+ *                  GAS_CHECK=1 is set, in which case the offsets are validated
+ *                  on the device first (with a stream synchronisation) and a
+ *                  violation returns GAS_ERROR_INVALID_VALUE with nothing sorted.
+ *   max_array_len > gas_max_array_len(): GAS_ERROR_UNSUPPORTED.
+ * One kernel launch per occupied size class (at most 12 launches).
+ */
+gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int64_t num_arrays,
+                                   int32_t max_array_len, cudaStream_t stream);
+
+/*
+ * Key + payload variant (north_star "optional key+payload variant"; SURVEY.md
+ * §8(f) row f2): keys as in gas_sort_arrays, d_values[i*n + j] is carried with
+ * d_keys[i*n + j]. STABLE: equal keys (identical bit patterns) keep their input
+ * order, so the payload order is unique (reading C-2). Same argument rules as
+ * gas_sort_arrays; both pointers 4-byte aligned.
+ */
+gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays, int32_t array_len,
+                          cudaStream_t stream);
+
+/*
+ * Host-memory convenience entry point (the paper's
+ * future-work out-of-core sort): h_data is HOST memory holding
+ * the fixed-length batch; it is streamed through the current device in
+ * chunks (host->device copy, sort, device->host copy on rotating streams so
+ * the two copy directions and the sort overlap) and the sorted batch is
+ * written back to h_data. Pinned (page-locked) host memory gives full-duplex
+ * PCIe; pageable memory works but is slower. BLOCKING: returns after the
+ * result is in h_data. Uses a stream-ordered device workspace of at most
+ * 3 x chunk (freed before return).
+ */
+gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array_len);
+
+/* Largest supported array length (4096: the paper's spectra bound). */
+int32_t gas_max_array_len(void);
+
+/* Static, human-readable name of a status code. */
+const char* gas_status_string(gas_status s);
+
+/* cudaError_t of the most recent GAS_ERROR_CUDA on this host thread (0 if none). */
+int gas_last_cuda_error(void);
+
+/* Number of kernels this library has launched in this process (monotone counter;
+   bench.py reports the delta over its timed region as "gpu_launches"). */
+int64_t gas_launch_count(void);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* GAS_H */

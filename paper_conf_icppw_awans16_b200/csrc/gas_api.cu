@@ -1,0 +1,250 @@
+// gas_api.cu — the C ABI of include/gas.h: argument validation, size-class
+// dispatch, launch configuration and status codes.
+#include <atomic>
+#include <cstdint>
+#include <cstdlib>
+#include <cstring>
+
+#include <cuda_runtime.h>
+
+#include "../../include/gas.h"
+#include "segsort.cuh"
+
+namespace {
+
+constexpr int32_t kMaxLen = 4096;  // spectra bound of P:L170-173, rounded to a size class
+
+thread_local int g_last_cuda_error = 0;
+std::atomic<int64_t> g_launches{0};
+
+gas_status cuda_fail(cudaError_t e) {
+  g_last_cuda_error = (int)e;
+  return GAS_ERROR_CUDA;
+}
+
+int num_sms() {
+  int dev = 0, sms = 0;
+  if (cudaGetDevice(&dev) != cudaSuccess) return 148;
+  if (cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev) != cudaSuccess || sms <= 0) return 148;
+  return sms;
+}
+
+int32_t size_class(int64_t n) {  // smallest power of two >= n, n >= 2
+  int32_t p = 2;
+  while (p < n) p <<= 1;
+  return p;
+}
+
+// Persistent grid: enough blocks to cover the work, at most the number of
+// blocks that can be resident on all SMs at once (a multiple of the SM count).
+template <typename K>
+int persistent_grid(K kernel, int threads, int64_t blocks_needed) {
+  int per_sm = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kernel, threads, 0) != cudaSuccess || per_sm <= 0)
+    per_sm = 1;
+  const int64_t cap = (int64_t)per_sm * num_sms();
+  return (int)(blocks_needed < cap ? (blocks_needed > 0 ? blocks_needed : 1) : cap);
+}
+
+template <int KPT, int G, bool VEC>
+cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  constexpr int arrays_per_block = (gas::kWarpBlock / 32) * (32 / G);
+  auto k = gas::k_fixed_warp<KPT, G, VEC>;
+  const int grid = persistent_grid(k, gas::kWarpBlock, (N + arrays_per_block - 1) / arrays_per_block);
+  k<<<grid, gas::kWarpBlock, 0, s>>>(d, N, n, 1u);
+  return cudaGetLastError();
+}
+
+template <int W, bool VEC>
+cudaError_t launch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  auto k = gas::k_fixed_cta<W, VEC>;
+  const int grid = persistent_grid(k, 32 * W, N);
+  k<<<grid, 32 * W, 0, s>>>(d, N, n, 1u);
+  return cudaGetLastError();
+}
+
+template <bool VEC>
+cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  switch (size_class(n)) {
+    case 2: return launch_fixed_warp<2, 1, false>(d, N, n, s);
+    case 4: return launch_fixed_warp<4, 1, VEC>(d, N, n, s);
+    case 8: return launch_fixed_warp<8, 1, VEC>(d, N, n, s);
+    case 16: return launch_fixed_warp<16, 1, VEC>(d, N, n, s);
+    case 32: return launch_fixed_warp<32, 1, VEC>(d, N, n, s);
+    case 64: return launch_fixed_warp<32, 2, VEC>(d, N, n, s);
+    case 128: return launch_fixed_warp<32, 4, VEC>(d, N, n, s);
+    case 256: return launch_fixed_warp<32, 8, VEC>(d, N, n, s);
+    case 512: return launch_fixed_warp<32, 16, VEC>(d, N, n, s);
+    case 1024: return launch_fixed_warp<32, 32, VEC>(d, N, n, s);
+    case 2048: return launch_fixed_cta<2, VEC>(d, N, n, s);
+    case 4096: return launch_fixed_cta<4, VEC>(d, N, n, s);
+  }
+  return cudaErrorInvalidValue;
+}
+
+template <int KPT, int G>
+cudaError_t launch_offsets_warp(uint32_t* d, const int64_t* off, int64_t N, cudaStream_t s) {
+  auto k = gas::k_offsets_warp<KPT, G>;
+  const int64_t windows = (N + 31) / 32;
+  const int grid = persistent_grid(k, gas::kWarpBlock, (windows + 7) / 8);
+  k<<<grid, gas::kWarpBlock, 0, s>>>(d, off, N, 1u);
+  return cudaGetLastError();
+}
+
+template <int W>
+cudaError_t launch_offsets_cta(uint32_t* d, const int64_t* off, int64_t N, cudaStream_t s) {
+  auto k = gas::k_offsets_cta<W>;
+  const int grid = persistent_grid(k, 32 * W, (N + 31) / 32);
+  k<<<grid, 32 * W, 0, s>>>(d, off, N, 1u);
+  return cudaGetLastError();
+}
+
+cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, int64_t N, cudaStream_t s) {
+  switch (P) {
+    case 2: return launch_offsets_warp<2, 1>(d, off, N, s);
+    case 4: return launch_offsets_warp<4, 1>(d, off, N, s);
+    case 8: return launch_offsets_warp<8, 1>(d, off, N, s);
+    case 16: return launch_offsets_warp<16, 1>(d, off, N, s);
+    case 32: return launch_offsets_warp<32, 1>(d, off, N, s);
+    case 64: return launch_offsets_warp<32, 2>(d, off, N, s);
+    case 128: return launch_offsets_warp<32, 4>(d, off, N, s);
+    case 256: return launch_offsets_warp<32, 8>(d, off, N, s);
+    case 512: return launch_offsets_warp<32, 16>(d, off, N, s);
+    case 1024: return launch_offsets_warp<32, 32>(d, off, N, s);
+    case 2048: return launch_offsets_cta<2>(d, off, N, s);
+    case 4096: return launch_offsets_cta<4>(d, off, N, s);
+  }
+  return cudaErrorInvalidValue;
+}
+
+// GAS_CHECK=1 validation of CSR offsets: flag = 1 on any violation.
+__global__ void k_check_offsets(const int64_t* __restrict__ off, int64_t N, int64_t max_len, int* flag) {
+  for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < N; i += (int64_t)gridDim.x * blockDim.x) {
+    const int64_t a = off[i], b = off[i + 1];
+    if (a < 0 || b < a || b - a > max_len) atomicOr(flag, 1);
+  }
+}
+
+bool env_check() {
+  const char* v = std::getenv("GAS_CHECK");
+  return v && std::strcmp(v, "0") != 0 && v[0] != '\0';
+}
+
+}  // namespace
+
+extern "C" {
+
+gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len, cudaStream_t stream) {
+  if (num_arrays < 0 || array_len < 0) return GAS_ERROR_INVALID_VALUE;
+  if (num_arrays == 0 || array_len <= 1) return GAS_SUCCESS;
+  if (array_len > kMaxLen) return GAS_ERROR_UNSUPPORTED;
+  if (d_data == nullptr || (reinterpret_cast<uintptr_t>(d_data) & 3u)) return GAS_ERROR_INVALID_VALUE;
+  uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
+  const bool vec = (reinterpret_cast<uintptr_t>(d_data) & 15u) == 0 && (array_len & 3) == 0;
+  const cudaError_t e = vec ? dispatch_fixed<true>(d, num_arrays, array_len, stream)
+                            : dispatch_fixed<false>(d, num_arrays, array_len, stream);
+  if (e != cudaSuccess) return cuda_fail(e);
+  g_launches.fetch_add(1, std::memory_order_relaxed);
+  return GAS_SUCCESS;
+}
+
+gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int64_t num_arrays,
+                                   int32_t max_array_len, cudaStream_t stream) {
+  if (num_arrays < 0 || max_array_len < 0) return GAS_ERROR_INVALID_VALUE;
+  if (max_array_len == 0) max_array_len = kMaxLen;
+  if (max_array_len > kMaxLen) return GAS_ERROR_UNSUPPORTED;
+  if (num_arrays == 0 || max_array_len <= 1) return GAS_SUCCESS;
+  if (d_offsets == nullptr || (reinterpret_cast<uintptr_t>(d_offsets) & 7u)) return GAS_ERROR_INVALID_VALUE;
+  if (d_data == nullptr || (reinterpret_cast<uintptr_t>(d_data) & 3u)) return GAS_ERROR_INVALID_VALUE;
+  if (env_check()) {
+    int* flag = nullptr;
+    cudaError_t e = cudaMallocAsync(&flag, sizeof(int), stream);
+    if (e != cudaSuccess) return cuda_fail(e);
+    int h = 0;
+    cudaMemsetAsync(flag, 0, sizeof(int), stream);
+    k_check_offsets<<<num_sms() * 4, 256, 0, stream>>>(d_offsets, num_arrays, max_array_len, flag);
+    g_launches.fetch_add(1, std::memory_order_relaxed);
+    cudaMemcpyAsync(&h, flag, sizeof(int), cudaMemcpyDeviceToHost, stream);
+    cudaFreeAsync(flag, stream);
+    e = cudaStreamSynchronize(stream);
+    if (e != cudaSuccess) return cuda_fail(e);
+    if (h) return GAS_ERROR_INVALID_VALUE;
+  }
+  uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
+  const int32_t top = size_class(max_array_len);
+  for (int32_t P = 2; P <= top; P <<= 1) {
+    const cudaError_t e = dispatch_offsets_class(P, d, d_offsets, num_arrays, stream);
+    if (e != cudaSuccess) return cuda_fail(e);
+    g_launches.fetch_add(1, std::memory_order_relaxed);
+  }
+  return GAS_SUCCESS;
+}
+
+gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays, int32_t array_len,
+                          cudaStream_t stream) {
+  (void)d_keys; (void)d_values; (void)num_arrays; (void)array_len; (void)stream;
+  return GAS_ERROR_UNSUPPORTED;
+}
+
+gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array_len) {
+  if (num_arrays < 0 || array_len < 0) return GAS_ERROR_INVALID_VALUE;
+  if (num_arrays == 0 || array_len <= 1) return GAS_SUCCESS;
+  if (array_len > kMaxLen) return GAS_ERROR_UNSUPPORTED;
+  if (h_data == nullptr || (reinterpret_cast<uintptr_t>(h_data) & 3u)) return GAS_ERROR_INVALID_VALUE;
+  constexpr int kSlots = 3;
+  constexpr int64_t kChunkBytes = 256ll << 20;
+  const int64_t row = (int64_t)array_len * 4;
+  int64_t per_chunk = kChunkBytes / row;
+  if (per_chunk < 1) per_chunk = 1;
+  if (per_chunk > num_arrays) per_chunk = num_arrays;
+  const int64_t nchunks = (num_arrays + per_chunk - 1) / per_chunk;
+  const int slots = (int)(nchunks < kSlots ? nchunks : kSlots);
+  cudaStream_t st[kSlots] = {};
+  float* buf[kSlots] = {};
+  gas_status status = GAS_SUCCESS;
+  cudaError_t e = cudaSuccess;
+  for (int s = 0; s < slots && e == cudaSuccess; ++s) {
+    e = cudaStreamCreateWithFlags(&st[s], cudaStreamNonBlocking);
+    if (e == cudaSuccess) e = cudaMalloc(&buf[s], per_chunk * row);
+  }
+  for (int64_t c = 0; c < nchunks && e == cudaSuccess && status == GAS_SUCCESS; ++c) {
+    const int s = (int)(c % slots);
+    const int64_t first = c * per_chunk;
+    const int64_t cnt = (first + per_chunk <= num_arrays) ? per_chunk : num_arrays - first;
+    float* h = h_data + first * array_len;
+    e = cudaMemcpyAsync(buf[s], h, cnt * row, cudaMemcpyHostToDevice, st[s]);
+    if (e != cudaSuccess) break;
+    status = gas_sort_arrays(buf[s], cnt, array_len, st[s]);
+    if (status != GAS_SUCCESS) break;
+    e = cudaMemcpyAsync(h, buf[s], cnt * row, cudaMemcpyDeviceToHost, st[s]);
+  }
+  for (int s = 0; s < slots; ++s) {
+    if (st[s]) {
+      const cudaError_t e2 = cudaStreamSynchronize(st[s]);
+      if (e == cudaSuccess) e = e2;
+      cudaStreamDestroy(st[s]);
+    }
+    if (buf[s]) cudaFree(buf[s]);
+  }
+  if (status != GAS_SUCCESS) return status;
+  if (e != cudaSuccess) return cuda_fail(e);
+  return GAS_SUCCESS;
+}
+
+int32_t gas_max_array_len(void) { return kMaxLen; }
+
+const char* gas_status_string(gas_status s) {
+  switch (s) {
+    case GAS_SUCCESS: return "GAS_SUCCESS";
+    case GAS_ERROR_INVALID_VALUE: return "GAS_ERROR_INVALID_VALUE";
+    case GAS_ERROR_UNSUPPORTED: return "GAS_ERROR_UNSUPPORTED";
+    case GAS_ERROR_CUDA: return "GAS_ERROR_CUDA";
+  }
+  return "GAS_UNKNOWN_STATUS";
+}
+
+int gas_last_cuda_error(void) { return g_last_cuda_error; }
+
+int64_t gas_launch_count(void) { return g_launches.load(std::memory_order_relaxed); }
+
+}  // extern "C"

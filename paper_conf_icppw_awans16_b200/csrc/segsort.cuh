@@ -1,0 +1,262 @@
+// segsort.cuh — the segment-sort kernels.
+//
+// One kernel instantiation per size class P = 2^p >= n (row a4). Each array
+// is owned by a group of G lanes (P <= 1024: several arrays per warp) or by a
+// CTA of W warps (P = 2048, 4096) — the paper's "each block is assigned one
+// array" at the granularity that fits the array. Per array:
+//   a2 stage in   HBM -> registers, coalesced (LDG.128 when 16-B aligned)
+//   a3 transform  float bits -> ordered uint32 key (ordered_key.cuh)
+//   a4 pad        slots n..P-1 = kPadKey
+//   a5 sort       bitonic network (bitonic.cuh)
+//   a6 inverse    key -> float bits
+//   a7 store      registers -> swizzled shared memory -> coalesced in-place
+//                 store (STG.128 when aligned); every byte is written once,
+//                 only inside the array's own range.
+// Kernels are persistent (grid-stride over arrays) so that the grid is a
+// multiple of the 148 SMs' resident blocks. Zero device workspace.
+#pragma once
+#include <cstdint>
+
+#include "bitonic.cuh"
+#include "ordered_key.cuh"
+
+namespace gas {
+
+constexpr int kWarpBlock = 256;  // threads per block for the warp-level classes
+
+// XOR swizzle of 16-byte chunks inside 128-byte rows: chunk c of a rank-order
+// buffer lives at physical chunk swz(c). Writes of 8 consecutive chunks per
+// thread and reads of 32 consecutive chunks per warp are both conflict-free.
+__device__ __forceinline__ int swz(int c) { return (c & ~7) | ((c ^ (c >> 3)) & 7); }
+
+__device__ __forceinline__ uint4 ld_stream(const uint4* p) { return __ldcs(p); }
+__device__ __forceinline__ uint32_t ld_stream(const uint32_t* p) { return __ldcs(p); }
+__device__ __forceinline__ void st_stream(uint4* p, uint4 v) { __stcs(p, v); }
+__device__ __forceinline__ void st_stream(uint32_t* p, uint32_t v) { __stcs(p, v); }
+
+// ---- a2-a4: load one array's n elements into KPT keys per thread ----------
+// Element (or 16-byte chunk) e of the array goes to thread (e % TH), slot
+// e / TH; which slot holds which input element is irrelevant to a sort.
+template <int KPT, int TH, bool VEC>
+__device__ __forceinline__ void load_keys(uint32_t (&k)[KPT], const uint32_t* __restrict__ src, int n, int tid,
+                                          bool valid) {
+  if constexpr (VEC) {
+    const uint4* s4 = reinterpret_cast<const uint4*>(src);
+    const int nc = n >> 2;
+#pragma unroll
+    for (int q = 0; q < KPT / 4; ++q) {
+      const int c = tid + TH * q;
+      uint4 v = make_uint4(kPadKey, kPadKey, kPadKey, kPadKey);
+      if (valid && c < nc) {
+        v = ld_stream(s4 + c);
+        v.x = key_from_bits(v.x); v.y = key_from_bits(v.y);
+        v.z = key_from_bits(v.z); v.w = key_from_bits(v.w);
+      }
+      k[4 * q + 0] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
+    }
+  } else {
+#pragma unroll
+    for (int q = 0; q < KPT; ++q) {
+      const int e = tid + TH * q;
+      k[q] = (valid && e < n) ? key_from_bits(ld_stream(src + e)) : kPadKey;
+    }
+  }
+}
+
+// ---- a6-a7 (part 1): thread holding ranks [tid*KPT, tid*KPT+KPT) writes
+// them, decoded, into the rank-order swizzled buffer `sb` (16-byte chunks).
+template <int KPT>
+__device__ __forceinline__ void stage_out(const uint32_t (&k)[KPT], uint4* sb, int chunk0) {
+  static_assert(KPT >= 4, "vector staging needs 4 keys per thread");
+#pragma unroll
+  for (int q = 0; q < KPT / 4; ++q)
+    sb[swz(chunk0 + q)] = make_uint4(bits_from_key(k[4 * q]), bits_from_key(k[4 * q + 1]),
+                                     bits_from_key(k[4 * q + 2]), bits_from_key(k[4 * q + 3]));
+}
+
+__device__ __forceinline__ uint32_t sword(const uint4* sb, int w) {
+  return reinterpret_cast<const uint32_t*>(sb)[swz(w >> 2) * 4 + (w & 3)];
+}
+__device__ __forceinline__ void sword_set(uint4* sb, int w, uint32_t v) {
+  reinterpret_cast<uint32_t*>(sb)[swz(w >> 2) * 4 + (w & 3)] = v;
+}
+
+// Write KPT rank-consecutive keys starting at rank-word w0 (any KPT).
+template <int KPT>
+__device__ __forceinline__ void stage_out_words(const uint32_t (&k)[KPT], uint4* sb, int w0) {
+  if constexpr (KPT >= 4) {
+    stage_out<KPT>(k, sb, w0 >> 2);
+  } else {
+#pragma unroll
+    for (int r = 0; r < KPT; ++r) sword_set(sb, w0 + r, bits_from_key(k[r]));
+  }
+}
+
+// ===================================================== fixed-length kernels
+
+// Warp-level classes: P = KPT * G <= 1024, GROUPS = 32 / G arrays per warp.
+template <int KPT, int G, bool VEC>
+__global__ void __launch_bounds__(kWarpBlock) k_fixed_warp(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+  constexpr int GROUPS = 32 / G;
+  constexpr int P = KPT * G;
+  constexpr int WORDS = 32 * KPT;  // per warp
+  __shared__ uint4 smem[kWarpBlock / 32][WORDS / 4 > 0 ? WORDS / 4 : 1];
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const int g = lane & (G - 1), grp = lane / G;
+  uint4* sb = smem[warp];
+  const int64_t nwarps = (int64_t)gridDim.x * (kWarpBlock / 32);
+  for (int64_t base = ((int64_t)blockIdx.x * (kWarpBlock / 32) + warp) * GROUPS; base < N; base += nwarps * GROUPS) {
+    const int64_t a = base + grp;
+    const bool valid = a < N;
+    uint32_t k[KPT];
+    load_keys<KPT, G, VEC>(k, d + (valid ? a : 0) * (int64_t)n, n, g, valid);
+    Bitonic<KPT, G, 1>::sort(k, g, 0, nullptr, one);
+    stage_out_words<KPT>(k, sb, grp * P + g * KPT);
+    __syncwarp();
+    if constexpr (VEC) {
+      // chunk c of the warp buffer = group c / (P/4), position (c % (P/4))*4
+      const int nc = n >> 2;
+#pragma unroll
+      for (int q = 0; q < KPT / 4; ++q) {
+        const int c = lane + 32 * q;
+        const int gg = c / (P / 4), pc = c % (P / 4);
+        const int64_t aa = base + gg;
+        if (aa < N && pc < nc) st_stream(reinterpret_cast<uint4*>(d + aa * (int64_t)n) + pc, sb[swz(c)]);
+      }
+    } else {
+#pragma unroll
+      for (int q = 0; q < KPT; ++q) {
+        const int w = lane + 32 * q;
+        const int gg = w / P, pw = w % P;
+        const int64_t aa = base + gg;
+        if (aa < N && pw < n) st_stream(d + aa * (int64_t)n + pw, sword(sb, w));
+      }
+    }
+    __syncwarp();
+  }
+}
+
+// CTA-level classes: P = 1024 * W (W = 2, 4), one array per CTA of 32W threads.
+template <int W, bool VEC>
+__global__ void __launch_bounds__(32 * W) k_fixed_cta(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+  constexpr int KPT = 32, T = 32 * W, P = KPT * T;
+  __shared__ uint4 smem[P / 4];
+  uint32_t* xs = reinterpret_cast<uint32_t*>(smem);
+  const int t = threadIdx.x, g = t & 31;
+  for (int64_t a = blockIdx.x; a < N; a += gridDim.x) {
+    uint32_t k[KPT];
+    load_keys<KPT, T, VEC>(k, d + a * (int64_t)n, n, t, true);
+    Bitonic<KPT, 32, W>::sort(k, g, t, xs, one);
+    __syncthreads();
+    stage_out_words<KPT>(k, smem, t * KPT);
+    __syncthreads();
+    if constexpr (VEC) {
+      const int nc = n >> 2;
+#pragma unroll
+      for (int q = 0; q < KPT / 4; ++q) {
+        const int c = t + T * q;
+        if (c < nc) st_stream(reinterpret_cast<uint4*>(d + a * (int64_t)n) + c, smem[swz(c)]);
+      }
+    } else {
+#pragma unroll
+      for (int q = 0; q < KPT; ++q) {
+        const int w = t + T * q;
+        if (w < n) st_stream(d + a * (int64_t)n + w, sword(smem, w));
+      }
+    }
+    __syncthreads();
+  }
+}
+
+// ===================================================== variable-length kernels
+// Array i = d[off[i] .. off[i+1]). A launch handles the arrays of one size
+// class (len in (P/2, P], or len == 2 for P == 2). Warps scan windows of 32
+// arrays, ballot the in-class ones and sort them GROUPS at a time, so that
+// no device workspace (index lists) is needed. Offsets may have any 4-byte
+// alignment, so loads/stores are scalar and masked to [off[i], off[i+1]).
+
+__device__ __forceinline__ bool in_class(int64_t len, int P) {
+  return P == 2 ? len == 2 : (len > P / 2 && len <= P);
+}
+
+template <int KPT, int G>
+__global__ void __launch_bounds__(kWarpBlock) k_offsets_warp(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
+                                                          int64_t N, uint32_t one) {
+  constexpr int GROUPS = 32 / G;
+  constexpr int P = KPT * G;
+  constexpr int WORDS = 32 * KPT;
+  __shared__ uint4 smem[kWarpBlock / 32][WORDS / 4 > 0 ? WORDS / 4 : 1];
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const int g = lane & (G - 1), grp = lane / G;
+  uint4* sb = smem[warp];
+  const int64_t nwarps = (int64_t)gridDim.x * (kWarpBlock / 32);
+  for (int64_t win = ((int64_t)blockIdx.x * (kWarpBlock / 32) + warp) * 32; win < N; win += nwarps * 32) {
+    const int64_t mine = win + lane;
+    int64_t my_lo = 0, my_len = 0;
+    if (mine < N) { my_lo = off[mine]; my_len = off[mine + 1] - my_lo; }
+    uint32_t mask = __ballot_sync(0xffffffffu, mine < N && in_class(my_len, P));
+    while (mask) {
+      const int cnt = __popc(mask);
+      const bool valid = grp < cnt;
+      const int pos = valid ? (int)__fns(mask, 0, grp + 1) : 0;
+      const int64_t lo = __shfl_sync(0xffffffffu, my_lo, pos);
+      const int len = (int)__shfl_sync(0xffffffffu, my_len, pos);
+      // the other groups' slots of this round, for the store phase
+      uint32_t k[KPT];
+      load_keys<KPT, G, false>(k, d + lo, len, g, valid);
+      Bitonic<KPT, G, 1>::sort(k, g, 0, nullptr, one);
+      stage_out_words<KPT>(k, sb, grp * P + g * KPT);
+      __syncwarp();
+#pragma unroll
+      for (int q = 0; q < KPT; ++q) {
+        const int w = lane + 32 * q;
+        const int gg = w / P, pw = w % P;
+        const int64_t glo = __shfl_sync(0xffffffffu, lo, gg * G);
+        const int glen = __shfl_sync(0xffffffffu, valid ? len : 0, gg * G);
+        if (pw < glen) st_stream(d + glo + pw, sword(sb, w));
+      }
+      __syncwarp();
+      if (cnt <= GROUPS) {
+        mask = 0;
+      } else {
+        const int last = (int)__fns(mask, 0, GROUPS);
+        mask &= (last >= 31) ? 0u : (0xffffffffu << (last + 1));
+      }
+    }
+  }
+}
+
+template <int W>
+__global__ void __launch_bounds__(32 * W) k_offsets_cta(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
+                                                        int64_t N, uint32_t one) {
+  constexpr int KPT = 32, T = 32 * W, P = KPT * T;
+  __shared__ uint4 smem[P / 4];
+  uint32_t* xs = reinterpret_cast<uint32_t*>(smem);
+  const int t = threadIdx.x, g = t & 31;
+  for (int64_t win = (int64_t)blockIdx.x * 32; win < N; win += (int64_t)gridDim.x * 32) {
+    const int64_t mine = win + g;
+    int64_t my_lo = 0, my_len = 0;
+    if (mine < N) { my_lo = off[mine]; my_len = off[mine + 1] - my_lo; }
+    uint32_t mask = __ballot_sync(0xffffffffu, mine < N && in_class(my_len, P));
+    while (mask) {  // identical in every warp of the CTA
+      const int pos = __ffs(mask) - 1;
+      mask &= mask - 1;
+      const int64_t lo = __shfl_sync(0xffffffffu, my_lo, pos);
+      const int len = (int)__shfl_sync(0xffffffffu, my_len, pos);
+      uint32_t k[KPT];
+      load_keys<KPT, T, false>(k, d + lo, len, t, true);
+      Bitonic<KPT, 32, W>::sort(k, g, t, xs, one);
+      __syncthreads();
+      stage_out_words<KPT>(k, smem, t * KPT);
+      __syncthreads();
+#pragma unroll
+      for (int q = 0; q < KPT; ++q) {
+        const int w = t + T * q;
+        if (w < len) st_stream(d + lo + w, sword(smem, w));
+      }
+      __syncthreads();
+    }
+  }
+}
+
+}  // namespace gas

@@ -1,0 +1,285 @@
+"""GPU parity: the CUDA path (through the C ABI) against the CPU oracle,
+element by element and bit-exact (the order is total on bit patterns, so the
+sorted output is unique — DESIGN.md reading C-2).
+
+Sizes span every size class (2 .. 4096), the tiles' ragged tails (n = 2^k±1,
+1000, 4000), zero and single arrays, unaligned base pointers (scalar path),
+non-default streams, canary words around the buffer, every input
+distribution; the full BASELINE.json configs[1] size (2M x 1000) is checked
+on sampled rows regenerated on the CPU plus whole-batch invariants."""
+import numpy as np
+import pytest
+
+import datagen
+import oracle
+
+torch = pytest.importorskip("torch")
+pytestmark = pytest.mark.gpu
+
+if not torch.cuda.is_available():  # pragma: no cover
+    pytest.skip("needs a GPU", allow_module_level=True)
+
+import paper_conf_icppw_awans16_b200 as gas  # noqa: E402
+
+DEV = torch.device("cuda:0")
+CANARY = np.uint32(0xDEADBEEF)
+
+
+def to_dev(a: np.ndarray) -> torch.Tensor:
+    return torch.from_numpy(np.ascontiguousarray(a).view(np.int32)).to(DEV)
+
+
+def to_host(t: torch.Tensor) -> np.ndarray:
+    return t.cpu().numpy().view(np.uint32)
+
+
+def gpu_sort_fixed(host: np.ndarray, lead: int = 4, stream=None) -> np.ndarray:
+    """Sort a [N, n] uint32 batch placed `lead` words into a canaried buffer."""
+    N, n = host.shape
+    buf = np.full(lead + N * n + 8, CANARY, dtype=np.uint32)
+    buf[lead:lead + N * n] = host.reshape(-1)
+    d = to_dev(buf)
+    ptr = d.data_ptr() + 4 * lead
+    s = stream if stream is not None else torch.cuda.current_stream()
+    gas.gas_sort_arrays_ptr(ptr, N, n, int(s.cuda_stream))
+    torch.cuda.synchronize()
+    out = to_host(d)
+    assert np.all(out[:lead] == CANARY) and np.all(out[lead + N * n:] == CANARY), "wrote outside the batch"
+    return out[lead:lead + N * n].reshape(N, n)
+
+
+def oracle_sorted(host: np.ndarray) -> np.ndarray:
+    e = host.copy()
+    oracle.sort_arrays_(e, threads=8)
+    return e
+
+
+SIZES = [2, 3, 4, 5, 7, 8, 9, 15, 16, 17, 31, 32, 33, 63, 64, 65, 100, 127, 128, 129, 255, 256, 257,
+         500, 511, 512, 513, 999, 1000, 1023, 1024, 1025, 1500, 2047, 2048, 2049, 3000, 4000, 4095, 4096]
+
+
+@pytest.mark.parametrize("n", SIZES)
+def test_every_size_class_uniform_bits(n):
+    N = max(3, min(300, 200000 // n))
+    host = datagen.fixed("uniform_bits", 101, 0, N, n)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=4), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("n", [4, 32, 100, 1000, 1024, 2000, 4000])
+def test_unaligned_base_scalar_path(n):
+    host = datagen.fixed("special_mix", 102, 0, 37, n)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=1), oracle_sorted(host))
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=3), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("dist", list(datagen.DISTS))
+@pytest.mark.parametrize("n", [1000, 4000, 333])
+def test_distributions(dist, n):
+    host = datagen.fixed(dist, datagen.config_seed(4), 0, 500 if n < 4000 else 120, n)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("N", [0, 1, 7, 1000])
+def test_batch_counts(N):
+    host = datagen.fixed("paper_uniform", datagen.config_seed(0), 0, N, 1000)
+    if N == 0:
+        t = torch.empty(0, 1000, dtype=torch.float32, device=DEV)
+        gas.gas_sort_arrays(t)
+        return
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+def test_config0_full_paper_uniform():
+    """BASELINE.json configs[0]: 1,000 arrays x 1,000 float32 uniform."""
+    host = datagen.fixed("paper_uniform", datagen.config_seed(0), 0, 1000, 1000)
+    x = torch.from_numpy(host.copy().view(np.float32)).to(DEV)
+    gas.gas_sort_arrays(x)
+    torch.cuda.synchronize()
+    np.testing.assert_array_equal(x.cpu().numpy().view(np.uint32), oracle_sorted(host))
+
+
+def test_nondefault_stream_and_tensor_api():
+    host = datagen.fixed("spectra_intensity", 5, 0, 999, 1000)
+    s = torch.cuda.Stream()
+    with torch.cuda.stream(s):
+        x = torch.from_numpy(host.copy().view(np.float32)).to(DEV, non_blocking=False)
+        gas.gas_sort_arrays(x)
+    s.synchronize()
+    np.testing.assert_array_equal(x.cpu().numpy().view(np.uint32), oracle_sorted(host))
+
+
+def test_zero_workspace():
+    x = torch.from_numpy(datagen.fixed("paper_uniform", 6, 0, 20000, 1000).view(np.float32)).to(DEV)
+    torch.cuda.synchronize()
+    free0, _ = torch.cuda.mem_get_info()
+    gas.gas_sort_arrays(x)
+    torch.cuda.synchronize()
+    free1, _ = torch.cuda.mem_get_info()
+    assert free1 == free0
+
+
+def test_idempotent_and_launch_count():
+    host = datagen.fixed("dup16", 7, 0, 300, 1000)
+    x = torch.from_numpy(host.copy().view(np.float32)).to(DEV)
+    c0 = gas.launch_count()
+    gas.gas_sort_arrays(x)
+    y = x.clone()
+    gas.gas_sort_arrays(y)
+    torch.cuda.synchronize()
+    assert gas.launch_count() == c0 + 2
+    assert torch.equal(x.view(torch.int32), y.view(torch.int32))
+
+
+# ------------------------------------------------------------ offsets variant
+
+
+def gpu_sort_offsets(data: np.ndarray, off: np.ndarray, lead: int = 3, max_len: int = 0):
+    buf = np.full(lead + data.size + 8, CANARY, dtype=np.uint32)
+    buf[lead:lead + data.size] = data
+    d = to_dev(buf)
+    # offsets relative to the buffer start (arrays begin `lead` words in)
+    o = torch.from_numpy(off + lead).to(DEV)
+    gas.gas_sort_arrays_offsets(d.view(torch.float32), o, max_len)
+    torch.cuda.synchronize()
+    out = to_host(d)
+    assert np.all(out[:lead] == CANARY) and np.all(out[lead + data.size:] == CANARY)
+    return out[lead:lead + data.size]
+
+
+@pytest.mark.parametrize("dist", ["uniform_bits", "special_mix", "paper_uniform", "dup16", "reverse"])
+def test_offsets_all_classes(dist):
+    lens = datagen.lengths(201, 0, 3000, 0, 4096)
+    lens[:12] = [0, 1, 2, 3, 4096, 0, 5, 4095, 1, 2049, 33, 1024]
+    off = datagen.offsets_from_lengths(lens)
+    data = datagen.ragged(dist, 201, 0, off)
+    expect = data.copy()
+    oracle.sort_arrays_offsets_(expect, off)
+    for lead in (0, 1, 2, 3):
+        np.testing.assert_array_equal(gpu_sort_offsets(data, off, lead=lead), expect)
+
+
+def test_offsets_spectra_lengths_config3_sample():
+    """BASELINE.json configs[3] recipe (lengths U{100..4000}) on 20k arrays."""
+    seed = datagen.config_seed(3)
+    lens = datagen.lengths(seed, 0, 20000, 100, 4000)
+    off = datagen.offsets_from_lengths(lens)
+    data = datagen.ragged("spectra_mz", seed, 0, off)
+    expect = data.copy()
+    oracle.sort_arrays_offsets_(expect, off)
+    np.testing.assert_array_equal(gpu_sort_offsets(data, off, lead=0, max_len=4000), expect)
+
+
+def test_offsets_with_gaps_between_arrays():
+    """Bytes between arrays (not covered by any [off[i], off[i+1])) are untouched:
+    CSR with repeated offsets gives empty arrays; gaps are modelled by sorting
+    only a sub-batch of a bigger buffer."""
+    lens = datagen.lengths(202, 0, 500, 0, 3000)
+    off = datagen.offsets_from_lengths(lens)
+    data = datagen.ragged("uniform_bits", 202, 0, off)
+    d = to_dev(data)
+    sub = torch.from_numpy(off[100:301].copy()).to(DEV)  # arrays 100..299 only
+    gas.gas_sort_arrays_offsets(d.view(torch.float32), sub)
+    torch.cuda.synchronize()
+    out = to_host(d)
+    expect = data.copy()
+    oracle.sort_arrays_offsets_(expect[off[100]:off[300]], off[100:301] - off[100])
+    np.testing.assert_array_equal(out, expect)
+
+
+def test_offsets_check_mode(monkeypatch):
+    monkeypatch.setenv("GAS_CHECK", "1")
+    data = to_dev(np.zeros(100, dtype=np.uint32)).view(torch.float32)
+    bad = torch.tensor([0, 50, 40, 100], dtype=torch.int64, device=DEV)
+    with pytest.raises(gas.GasError):
+        gas.gas_sort_arrays_offsets(data, bad)
+    too_long = torch.tensor([0, 100], dtype=torch.int64, device=DEV)
+    with pytest.raises(gas.GasError):
+        gas.gas_sort_arrays_offsets(data, too_long, 64)
+    ok = torch.tensor([0, 60, 100], dtype=torch.int64, device=DEV)
+    gas.gas_sort_arrays_offsets(data, ok)
+
+
+# ------------------------------------------------------------ host entry point
+
+
+@pytest.mark.parametrize("N,n", [(5000, 1000), (333, 4000), (10, 7)])
+def test_host_entry_point(N, n):
+    host = datagen.fixed("special_mix", 301, 0, N, n)
+    h = torch.from_numpy(host.copy().view(np.float32)).pin_memory()
+    gas.gas_sort_arrays_host(h)
+    np.testing.assert_array_equal(h.numpy().view(np.uint32), oracle_sorted(host))
+
+
+def test_host_entry_point_many_chunks():
+    # > 3 chunks of 256 MB: 300k x 1000 floats = 1.2 GB
+    N, n = 300000, 1000
+    h = torch.empty(N, n, dtype=torch.float32).pin_memory()
+    d = torch.empty(N, n, dtype=torch.float32, device=DEV)
+    datagen.fixed_device(d, "paper_uniform", 9, 0, N, n)
+    h.copy_(d.cpu())
+    gas.gas_sort_arrays_host(h)
+    rows = np.random.default_rng(0).choice(N, 300, replace=False)
+    expect = oracle_sorted(datagen.rows("paper_uniform", 9, rows, n))
+    np.testing.assert_array_equal(h.numpy().view(np.uint32)[rows], expect)
+
+
+# ------------------------------------------------------------ generator twin
+
+
+@pytest.mark.parametrize("dist", list(datagen.DISTS))
+def test_device_generator_matches_numpy(dist):
+    N, n = 97, 1001
+    d = torch.empty(N * n, dtype=torch.int32, device=DEV)
+    datagen.fixed_device(d, dist, 77, 13, N, n)
+    torch.cuda.synchronize()
+    np.testing.assert_array_equal(to_host(d).reshape(N, n), datagen.fixed(dist, 77, 13, N, n))
+    lens = datagen.lengths(78, 0, 200, 0, 700)
+    off = datagen.offsets_from_lengths(lens)
+    r = torch.empty(int(off[-1]), dtype=torch.int32, device=DEV)
+    datagen.ragged_device(r, torch.from_numpy(off).to(DEV), dist, 78, 5, len(lens))
+    torch.cuda.synchronize()
+    np.testing.assert_array_equal(to_host(r), datagen.ragged(dist, 78, 5, off))
+
+
+# ------------------------------------------------------------ full-size config
+
+
+def _row_keys_sorted(x: torch.Tensor) -> bool:
+    """All rows nondecreasing under the ordered-key view (computed with torch int64)."""
+    ok = True
+    for lo in range(0, x.shape[0], 100000):
+        b = x[lo:lo + 100000].view(torch.int32).to(torch.int64) & 0xFFFFFFFF
+        neg = (b >> 31) == 1
+        k = torch.where(neg, b ^ 0xFFFFFFFF, b ^ 0x80000000)
+        ok &= bool((k[:, 1:] >= k[:, :-1]).all())
+    return ok
+
+
+def _row_checksums(x: torch.Tensor):
+    out = []
+    for lo in range(0, x.shape[0], 100000):
+        b = x[lo:lo + 100000].view(torch.int32).to(torch.int64) & 0xFFFFFFFF
+        out.append(torch.stack([b.sum(1), (b * b % 1000003).sum(1), (b ^ (b >> 7)).sum(1)], 1))
+    return torch.cat(out)
+
+
+@pytest.mark.parametrize("dist", ["paper_uniform", "special_mix"])
+def test_config1_full_size_sampled(dist):
+    """BASELINE.json configs[1]: 2,000,000 x 1,000 in the bench's launch
+    configuration; 2,000 sampled rows bit-exact vs the oracle, all rows
+    sorted and permutation-checksummed."""
+    N, n = 2_000_000, 1000
+    seed = datagen.config_seed(1)
+    x = torch.empty(N, n, dtype=torch.float32, device=DEV)
+    datagen.fixed_device(x, dist, seed, 0, N, n)
+    ck0 = _row_checksums(x)
+    gas.gas_sort_arrays(x)
+    torch.cuda.synchronize()
+    assert _row_keys_sorted(x)
+    assert torch.equal(ck0, _row_checksums(x))
+    rows = np.sort(np.random.default_rng(1).choice(N, 2000, replace=False))
+    rows[-1] = N - 1
+    rows[0] = 0
+    expect = oracle_sorted(datagen.rows(dist, seed, rows, n))
+    got = x[torch.from_numpy(rows).to(DEV)].view(torch.int32).cpu().numpy().view(np.uint32)
+    np.testing.assert_array_equal(got, expect)
