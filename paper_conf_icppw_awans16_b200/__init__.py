@@ -19,7 +19,7 @@ import ctypes
 import os
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libgas.so")
+LIB_PATH = os.environ.get("GAS_LIB") or os.path.join(_HERE, "libgas.so")  # GAS_LIB: experiment builds
 
 GAS_SUCCESS = 0
 GAS_ERROR_INVALID_VALUE = 1

@@ -19,10 +19,14 @@
 
 #include "bitonic.cuh"
 #include "ordered_key.cuh"
+#include "warp1024.cuh"
 
 namespace gas {
 
 constexpr int kWarpBlock = 256;  // threads per block for the warp-level classes
+#ifndef GAS_WARP_MIN_BLOCKS
+#define GAS_WARP_MIN_BLOCKS 2     // 2 x 256 threads = 16 warps/SM -> up to 128 registers (no spills)
+#endif
 
 // XOR swizzle of 16-byte chunks inside 128-byte rows: chunk c of a rank-order
 // buffer lives at physical chunk swz(c). Writes of 8 consecutive chunks per
@@ -96,7 +100,7 @@ __device__ __forceinline__ void stage_out_words(const uint32_t (&k)[KPT], uint4*
 
 // Warp-level classes: P = KPT * G <= 1024, GROUPS = 32 / G arrays per warp.
 template <int KPT, int G, bool VEC>
-__global__ void __launch_bounds__(kWarpBlock) k_fixed_warp(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+__global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS) k_fixed_warp(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   constexpr int GROUPS = 32 / G;
   constexpr int P = KPT * G;
   constexpr int WORDS = 32 * KPT;  // per warp
@@ -110,7 +114,8 @@ __global__ void __launch_bounds__(kWarpBlock) k_fixed_warp(uint32_t* __restrict_
     const bool valid = a < N;
     uint32_t k[KPT];
     load_keys<KPT, G, VEC>(k, d + (valid ? a : 0) * (int64_t)n, n, g, valid);
-    Bitonic<KPT, G, 1>::sort(k, g, 0, nullptr, one);
+    if constexpr (KPT == 32 && G == 32) sort1024_warp(k, lane, reinterpret_cast<uint32_t*>(sb), one);
+    else Bitonic<KPT, G, 1>::sort(k, g, 0, nullptr, one);
     stage_out_words<KPT>(k, sb, grp * P + g * KPT);
     __syncwarp();
     if constexpr (VEC) {
