@@ -245,8 +245,10 @@ def main():
         if pg:
             pg.barrier()
 
+    from paper_conf_icppw_awans16_b200 import shard
+
     N_rank = cfg["N"]
-    i0 = rank * N_rank  # weak scaling: rank r owns arrays [r*N, (r+1)*N) of the global stream
+    i0, _ = shard.weak_range(N_rank, rank)  # weak scaling: rank r owns arrays [r*N, (r+1)*N)
     stream = torch.cuda.current_stream()
     ragged = cfg["n"] is None
     if ragged:
@@ -296,11 +298,7 @@ def main():
     barrier()
     launches = gas.launch_count() - launches0
     per_step = [a.elapsed_time(b) for a, b in evs]
-    t_sum = sum(per_step)
-    if pg:
-        t = torch.tensor([t_sum], dtype=torch.float64, device=dev)
-        pg.all_reduce(t, op=pg.ReduceOp.MAX)
-        t_sum = float(t.item())
+    t_sum = shard.max_over_ranks(sum(per_step), dev)  # the slowest rank defines the job
     ms_per_step = t_sum / args.steps
     total_arrays = N_rank * world
     value = total_arrays / (ms_per_step * 1e-3)
@@ -328,12 +326,7 @@ def main():
             dt = time.perf_counter() - t0
             if s > 0:
                 ts.append(dt)
-        if pg:
-            t = torch.tensor([sum(ts)], dtype=torch.float64, device=dev)
-            pg.all_reduce(t, op=pg.ReduceOp.MAX)
-            dt = float(t.item()) / len(ts)
-        else:
-            dt = sum(ts) / len(ts)
+        dt = shard.max_over_ranks(sum(ts), dev) / len(ts)
         nbytes = N_rank * cfg["n"] * 4
         e2e = {"value": total_arrays / dt, "unit": "arrays/s", "h2d_bytes_per_step": nbytes,
                "d2h_bytes_per_step": nbytes, "ms_per_step": dt * 1e3,
