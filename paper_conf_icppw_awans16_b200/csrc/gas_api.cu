@@ -63,6 +63,27 @@ cudaError_t launch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   return cudaGetLastError();
 }
 
+bool env_flag(const char* name) {
+  const char* v = std::getenv(name);
+  return v && v[0] != '\0' && std::strcmp(v, "0") != 0;
+}
+
+cudaError_t launch_fixed_1024_tma(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  // per-device attribute: set on every call (cheap), the current device may change
+  const cudaError_t attr = cudaFuncSetAttribute(gas::k_fixed_1024_tma, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                                gas::kTmaSmemBytes);
+  if (attr != cudaSuccess) return attr;
+  int per_sm = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, gas::k_fixed_1024_tma, gas::kWarpBlock,
+                                                    gas::kTmaSmemBytes) != cudaSuccess || per_sm <= 0)
+    per_sm = 1;
+  const int64_t need = (N + gas::kWarpBlock / 32 - 1) / (gas::kWarpBlock / 32);
+  const int64_t cap = (int64_t)per_sm * num_sms();
+  const int grid = (int)(need < cap ? need : cap);
+  gas::k_fixed_1024_tma<<<grid, gas::kWarpBlock, gas::kTmaSmemBytes, s>>>(d, N, n, 1u);
+  return cudaGetLastError();
+}
+
 template <bool VEC>
 cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   switch (size_class(n)) {
@@ -75,7 +96,12 @@ cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
     case 128: return launch_fixed_warp<32, 4, VEC>(d, N, n, s);
     case 256: return launch_fixed_warp<32, 8, VEC>(d, N, n, s);
     case 512: return launch_fixed_warp<32, 16, VEC>(d, N, n, s);
-    case 1024: return launch_fixed_warp<32, 32, VEC>(d, N, n, s);
+    case 1024:
+      // TMA-prefetch variant: opt-in (GAS_TMA=1). Measured on B200 it removes the
+      // global-load stalls but is 5% slower overall (profiles/r01_ab_tma.txt):
+      // the kernel is ALU/issue-bound, not latency-bound.
+      if (VEC && env_flag("GAS_TMA")) return launch_fixed_1024_tma(d, N, n, s);
+      return launch_fixed_warp<32, 32, VEC>(d, N, n, s);
     case 2048: return launch_fixed_cta<2, VEC>(d, N, n, s);
     case 4096: return launch_fixed_cta<4, VEC>(d, N, n, s);
   }

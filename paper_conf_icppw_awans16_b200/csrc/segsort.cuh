@@ -20,6 +20,7 @@
 #include "bitonic.cuh"
 #include "ordered_key.cuh"
 #include "warp1024.cuh"
+#include "bulk.cuh"
 
 namespace gas {
 
@@ -137,6 +138,69 @@ __global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS) k_fixed_warp(
         if (aa < N && pw < n) st_stream(d + aa * (int64_t)n + pw, sword(sb, w));
       }
     }
+    __syncwarp();
+  }
+}
+
+// P = 1024 class with 16-byte-aligned rows (n % 4 == 0, aligned base): one
+// warp per array; while the warp sorts array t its next array t+1 is already
+// in flight into the warp's second shared-memory buffer by a TMA bulk copy
+// (cp.async.bulk + mbarrier), so global-load latency is off the critical
+// path. Dynamic shared memory: kWarpBlock/32 warps x 2 x 4 KB + barriers.
+constexpr int kTmaSmemBytes = (kWarpBlock / 32) * 2 * 4096 + (kWarpBlock / 32) * 2 * 8;
+
+__global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS)
+    k_fixed_1024_tma(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+  extern __shared__ __align__(128) uint4 dsm[];
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  uint4* buf0 = dsm + warp * 512;  // 2 x 256 uint4 per warp
+  uint64_t* bar = reinterpret_cast<uint64_t*>(dsm + (kWarpBlock / 32) * 512) + warp * 2;
+  const int64_t nwarps = (int64_t)gridDim.x * (kWarpBlock / 32);
+  int64_t a = (int64_t)blockIdx.x * (kWarpBlock / 32) + warp;
+  const uint32_t bytes = (uint32_t)n * 4u;
+  const int nc = n >> 2;
+  if (lane == 0) {
+    mbar_init(&bar[0], 1);
+    mbar_init(&bar[1], 1);
+    fence_mbar_init();
+    if (a < N) {
+      mbar_arrive_expect_tx(&bar[0], bytes);
+      bulk_g2s(buf0, d + a * (int64_t)n, bytes, &bar[0]);
+    }
+  }
+  __syncwarp();
+  for (uint32_t t = 0; a < N; ++t, a += nwarps) {
+    const uint32_t b = t & 1u;
+    uint4* cur = buf0 + b * 256;
+    const int64_t an = a + nwarps;
+    if (lane == 0 && an < N) {  // prefetch the next array into the other buffer
+      mbar_arrive_expect_tx(&bar[b ^ 1u], bytes);
+      bulk_g2s(buf0 + (b ^ 1u) * 256, d + an * (int64_t)n, bytes, &bar[b ^ 1u]);
+    }
+    mbar_wait_parity(&bar[b], (t >> 1) & 1u);
+    uint32_t k[32];
+#pragma unroll
+    for (int q = 0; q < 8; ++q) {
+      const int c = lane + 32 * q;
+      uint4 v = make_uint4(kPadKey, kPadKey, kPadKey, kPadKey);
+      if (c < nc) {
+        v = cur[c];
+        v.x = key_from_bits(v.x); v.y = key_from_bits(v.y);
+        v.z = key_from_bits(v.z); v.w = key_from_bits(v.w);
+      }
+      k[4 * q + 0] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
+    }
+    __syncwarp();  // every lane has its data: the buffer becomes sort scratch
+    sort1024_warp(k, lane, reinterpret_cast<uint32_t*>(cur), one);
+    stage_out<32>(k, cur, lane * 8);
+    __syncwarp();
+    uint4* dst = reinterpret_cast<uint4*>(d + a * (int64_t)n);
+#pragma unroll
+    for (int q = 0; q < 8; ++q) {
+      const int c = lane + 32 * q;
+      if (c < nc) st_stream(dst + c, cur[swz(c)]);
+    }
+    fence_proxy_async_smem();  // generic reads of `cur` before the next bulk write into it
     __syncwarp();
   }
 }
