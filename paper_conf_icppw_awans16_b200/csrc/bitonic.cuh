@@ -63,12 +63,22 @@ __device__ __forceinline__ void ce_n(int c, uint32_t& a, uint32_t& b, uint32_t o
   else ce<false>(a, b, one);
 }
 
+// 64-bit elements (key << 32 | original position: the stable pairs variant).
+__device__ __forceinline__ void ce_n(int, uint64_t& a, uint64_t& b, uint32_t) {
+  const uint64_t mn = a < b ? a : b;
+  b = a < b ? b : a;
+  a = mn;
+}
+
 // Keep the min (lower index) or the max (upper index) of x and the partner's y.
 __device__ __forceinline__ uint32_t keep(uint32_t x, uint32_t y, bool upper) {
   return upper ? max(x, y) : min(x, y);
 }
+__device__ __forceinline__ uint64_t keep(uint64_t x, uint64_t y, bool upper) {
+  return (upper == (x < y)) ? y : x;
+}
 
-template <int KPT, int G, int W>
+template <int KPT, int G, int W, typename T = uint32_t>
 struct Bitonic {
   static_assert(KPT >= 1 && (KPT & (KPT - 1)) == 0, "KPT power of two");
   static_assert(G >= 1 && G <= 32 && (G & (G - 1)) == 0, "G power of two <= 32");
@@ -77,11 +87,11 @@ struct Bitonic {
   static constexpr int LOGG = Log2<G>::value;
   static constexpr int P = KPT * G * W;
   static constexpr int LOGP = Log2<P>::value;
-  static constexpr int T = 32 * W;  // threads per array when W > 1
+  static constexpr int NT = 32 * W;  // threads per array when W > 1
 
   // In-register stage at distance j (< KPT): pairs (r, r|j) with bit j clear.
   template <int J>
-  __device__ __forceinline__ static void reg_stage(uint32_t (&k)[KPT], uint32_t one) {
+  __device__ __forceinline__ static void reg_stage(T (&k)[KPT], uint32_t one) {
 #pragma unroll
     for (int r = 0; r < KPT; ++r)
       if (!(r & J)) ce_n(r, k[r], k[r | J], one);
@@ -89,7 +99,7 @@ struct Bitonic {
 
   // In-register mirror stage of merge size K (<= KPT): pairs (r, r ^ (K-1)).
   template <int K>
-  __device__ __forceinline__ static void reg_mirror(uint32_t (&k)[KPT], uint32_t one) {
+  __device__ __forceinline__ static void reg_mirror(T (&k)[KPT], uint32_t one) {
 #pragma unroll
     for (int r = 0; r < KPT; ++r)
       if (!(r & (K / 2))) ce_n(r, k[r], k[r ^ (K - 1)], one);
@@ -97,19 +107,19 @@ struct Bitonic {
 
   // Shared-memory exchange stage for partners in other warps. Element (t, r)
   // is stored at xs[r*T + t] (conflict-free for consecutive t).
-  __device__ __forceinline__ static void smem_stage(uint32_t (&k)[KPT], uint32_t* xs, int t, int tmask,
+  __device__ __forceinline__ static void smem_stage(T (&k)[KPT], T* xs, int t, int tmask,
                                                     int rmask, bool upper) {
     __syncthreads();
 #pragma unroll
-    for (int r = 0; r < KPT; ++r) xs[r * T + t] = k[r];
+    for (int r = 0; r < KPT; ++r) xs[r * NT + t] = k[r];
     __syncthreads();
 #pragma unroll
-    for (int r = 0; r < KPT; ++r) k[r] = keep(k[r], xs[(r ^ rmask) * T + (t ^ tmask)], upper);
+    for (int r = 0; r < KPT; ++r) k[r] = keep(k[r], xs[(r ^ rmask) * NT + (t ^ tmask)], upper);
   }
 
   // Half-cleaner at distance 2^LJ, then the rest of the cascade down to 1.
   template <int LJ>
-  __device__ __forceinline__ static void cleaners(uint32_t (&k)[KPT], int g, int t, uint32_t* xs, uint32_t one) {
+  __device__ __forceinline__ static void cleaners(T (&k)[KPT], int g, int t, T* xs, uint32_t one) {
     if constexpr (LJ >= 0) {
       constexpr int J = 1 << LJ;
       if constexpr (LJ < LOGK) {
@@ -128,7 +138,7 @@ struct Bitonic {
 
   // Merge step of size K = 2^LK: mirror stage (partner i ^ (K-1)), then cleaners.
   template <int LK>
-  __device__ __forceinline__ static void merge(uint32_t (&k)[KPT], int g, int t, uint32_t* xs, uint32_t one) {
+  __device__ __forceinline__ static void merge(T (&k)[KPT], int g, int t, T* xs, uint32_t one) {
     constexpr int K = 1 << LK;
     if constexpr (LK <= LOGK) {
       reg_mirror<K>(k, one);
@@ -141,8 +151,8 @@ struct Bitonic {
 #pragma unroll
         for (int r = 0; r < KPT / 2; ++r) {
           const int r2 = KPT - 1 - r;
-          const uint32_t v1 = __shfl_xor_sync(0xffffffffu, k[r2], m);
-          const uint32_t v2 = __shfl_xor_sync(0xffffffffu, k[r], m);
+          const T v1 = __shfl_xor_sync(0xffffffffu, k[r2], m);
+          const T v2 = __shfl_xor_sync(0xffffffffu, k[r], m);
           k[r] = keep(k[r], v1, upper);
           k[r2] = keep(k[r2], v2, upper);
         }
@@ -154,7 +164,7 @@ struct Bitonic {
   }
 
   template <int LK>
-  __device__ __forceinline__ static void sort_from(uint32_t (&k)[KPT], int g, int t, uint32_t* xs, uint32_t one) {
+  __device__ __forceinline__ static void sort_from(T (&k)[KPT], int g, int t, T* xs, uint32_t one) {
     if constexpr (LK <= LOGP) {
       merge<LK>(k, g, t, xs, one);
       sort_from<LK + 1>(k, g, t, xs, one);
@@ -164,7 +174,7 @@ struct Bitonic {
   // Sort the P keys ascending. g: lane index inside the G-lane group;
   // t: thread index inside the array's W warps (t = w*32 + g; used when W > 1);
   // xs: P words of shared memory (used when W > 1).
-  __device__ __forceinline__ static void sort(uint32_t (&k)[KPT], int g, int t, uint32_t* xs, uint32_t one) {
+  __device__ __forceinline__ static void sort(T (&k)[KPT], int g, int t, T* xs, uint32_t one) {
     sort_from<1>(k, g, t, xs, one);
   }
 };

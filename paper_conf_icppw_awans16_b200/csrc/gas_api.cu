@@ -9,6 +9,7 @@
 
 #include "../../include/gas.h"
 #include "segsort.cuh"
+#include "pairs.cuh"
 
 namespace {
 
@@ -143,6 +144,39 @@ cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, i
   return cudaErrorInvalidValue;
 }
 
+template <int KPT, int G, int W>
+cudaError_t launch_pairs(uint32_t* k, uint32_t* v, int64_t N, int n, cudaStream_t s) {
+  using C = gas::PairsCfg<KPT, G, W>;
+  auto kern = gas::k_pairs<KPT, G, W>;
+  cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
+  if (e != cudaSuccess) return e;
+  int per_sm = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, C::TPB, C::SMEM) != cudaSuccess || per_sm <= 0)
+    per_sm = 1;
+  const int64_t need = (N + C::GROUPS - 1) / C::GROUPS;
+  const int64_t cap = (int64_t)per_sm * num_sms();
+  kern<<<(int)(need < cap ? need : cap), C::TPB, C::SMEM, s>>>(k, v, N, n);
+  return cudaGetLastError();
+}
+
+cudaError_t dispatch_pairs(uint32_t* k, uint32_t* v, int64_t N, int n, cudaStream_t s) {
+  switch (size_class(n)) {
+    case 2: return launch_pairs<2, 1, 1>(k, v, N, n, s);
+    case 4: return launch_pairs<4, 1, 1>(k, v, N, n, s);
+    case 8: return launch_pairs<8, 1, 1>(k, v, N, n, s);
+    case 16: return launch_pairs<16, 1, 1>(k, v, N, n, s);
+    case 32: return launch_pairs<32, 1, 1>(k, v, N, n, s);
+    case 64: return launch_pairs<32, 2, 1>(k, v, N, n, s);
+    case 128: return launch_pairs<32, 4, 1>(k, v, N, n, s);
+    case 256: return launch_pairs<32, 8, 1>(k, v, N, n, s);
+    case 512: return launch_pairs<32, 16, 1>(k, v, N, n, s);
+    case 1024: return launch_pairs<32, 32, 1>(k, v, N, n, s);
+    case 2048: return launch_pairs<32, 32, 2>(k, v, N, n, s);
+    case 4096: return launch_pairs<32, 32, 4>(k, v, N, n, s);
+  }
+  return cudaErrorInvalidValue;
+}
+
 // GAS_CHECK=1 validation of CSR offsets: flag = 1 on any violation.
 __global__ void k_check_offsets(const int64_t* __restrict__ off, int64_t N, int64_t max_len, int* flag) {
   for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < N; i += (int64_t)gridDim.x * blockDim.x) {
@@ -208,8 +242,16 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
 
 gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays, int32_t array_len,
                           cudaStream_t stream) {
-  (void)d_keys; (void)d_values; (void)num_arrays; (void)array_len; (void)stream;
-  return GAS_ERROR_UNSUPPORTED;
+  if (num_arrays < 0 || array_len < 0) return GAS_ERROR_INVALID_VALUE;
+  if (num_arrays == 0 || array_len <= 1) return GAS_SUCCESS;
+  if (array_len > kMaxLen) return GAS_ERROR_UNSUPPORTED;
+  if (d_keys == nullptr || d_values == nullptr || (reinterpret_cast<uintptr_t>(d_keys) & 3u) ||
+      (reinterpret_cast<uintptr_t>(d_values) & 3u))
+    return GAS_ERROR_INVALID_VALUE;
+  const cudaError_t e = dispatch_pairs(reinterpret_cast<uint32_t*>(d_keys), d_values, num_arrays, array_len, stream);
+  if (e != cudaSuccess) return cuda_fail(e);
+  g_launches.fetch_add(1, std::memory_order_relaxed);
+  return GAS_SUCCESS;
 }
 
 gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array_len) {

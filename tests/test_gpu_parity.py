@@ -283,3 +283,35 @@ def test_config1_full_size_sampled(dist):
     expect = oracle_sorted(datagen.rows(dist, seed, rows, n))
     got = x[torch.from_numpy(rows).to(DEV)].view(torch.int32).cpu().numpy().view(np.uint32)
     np.testing.assert_array_equal(got, expect)
+
+
+# ------------------------------------------------------------ stable pairs (f2)
+
+
+@pytest.mark.parametrize("n", [2, 3, 16, 33, 100, 512, 1000, 1024, 1500, 2048, 4000, 4096])
+@pytest.mark.parametrize("dist", ["dup16", "special_mix", "uniform_bits"])
+def test_pairs_stable_vs_oracle(n, dist):
+    N = max(3, min(200, 100000 // n))
+    keys = datagen.fixed(dist, 401, 0, N, n)
+    vals = datagen.fixed("uniform_bits", 402, 0, N, n)
+    kd, vd = to_dev(keys), to_dev(vals)
+    gas.gas_sort_pairs(kd.view(torch.float32), vd)
+    torch.cuda.synchronize()
+    ek, ev = keys.copy(), vals.copy()
+    oracle.sort_pairs_(ek, ev)
+    np.testing.assert_array_equal(to_host(kd).reshape(N, n), ek)
+    np.testing.assert_array_equal(to_host(vd).reshape(N, n), ev)
+
+
+def test_pairs_payload_is_original_position():
+    N, n = 300, 1000
+    keys = datagen.fixed("dup16", 403, 0, N, n)
+    pos = np.tile(np.arange(n, dtype=np.uint32), (N, 1))
+    kd, vd = to_dev(keys), to_dev(pos)
+    gas.gas_sort_pairs(kd.view(torch.float32), vd)
+    torch.cuda.synchronize()
+    k, v = to_host(kd).reshape(N, n), to_host(vd).reshape(N, n)
+    for i in range(0, N, 37):
+        np.testing.assert_array_equal(keys[i][v[i]], k[i])
+        for kv in np.unique(k[i]):
+            assert np.all(np.diff(v[i][k[i] == kv].astype(np.int64)) > 0)
