@@ -45,6 +45,8 @@ def parse():
     p.add_argument("--warmup", type=int, default=3)
     p.add_argument("--config", type=int, default=1, choices=sorted(CONFIGS))
     p.add_argument("--dist", default=None, help="override the config's value distribution")
+    p.add_argument("--n", type=int, default=None, help="override the array length (fixed-length configs)")
+    p.add_argument("--arrays", type=int, default=None, help="override the number of arrays per GPU")
     p.add_argument("--impl", default="gas", choices=["gas", "reference"])
     p.add_argument("--no-e2e", action="store_true")
     p.add_argument("--no-cpu-baseline", action="store_true")
@@ -221,7 +223,13 @@ def reference_arm(args, cfg, dist, seed):
 
 def main():
     args = parse()
-    cfg = CONFIGS[args.config]
+    cfg = dict(CONFIGS[args.config])
+    if args.n is not None or args.arrays is not None:
+        if args.n is not None:
+            cfg["n"] = args.n
+        if args.arrays is not None:
+            cfg["N"] = args.arrays
+        cfg["name"] = f"custom sweep from configs[{args.config}]: {cfg['N']:,} arrays x {cfg['n']} float32"
     dist = args.dist or cfg["dist"]
     import datagen
 

@@ -76,7 +76,8 @@ gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len,
  *                  on the device first (with a stream synchronisation) and a
  *                  violation returns GAS_ERROR_INVALID_VALUE with nothing sorted.
  *   max_array_len > gas_max_array_len(): GAS_ERROR_UNSUPPORTED.
- * One kernel launch per occupied size class (at most 12 launches).
+ * One kernel launch per size class up to max_array_len (at most 13 launches:
+ * powers of two up to 2048, then (2048, 3072] and (3072, 4096]).
  */
 gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int64_t num_arrays,
                                    int32_t max_array_len, cudaStream_t stream);

@@ -56,11 +56,11 @@ cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   return cudaGetLastError();
 }
 
-template <int W, bool VEC>
+template <int W, int WR, bool VEC>
 cudaError_t launch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  auto k = gas::k_fixed_cta<W, VEC>;
-  const int grid = persistent_grid(k, 32 * W, N);
-  k<<<grid, 32 * W, 0, s>>>(d, N, n, 1u);
+  auto k = gas::k_fixed_cta<W, WR, VEC>;
+  const int grid = persistent_grid(k, 32 * WR, N);
+  k<<<grid, 32 * WR, 0, s>>>(d, N, n, 1u);
   return cudaGetLastError();
 }
 
@@ -103,8 +103,9 @@ cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
       // the kernel is ALU/issue-bound, not latency-bound.
       if (VEC && env_flag("GAS_TMA")) return launch_fixed_1024_tma(d, N, n, s);
       return launch_fixed_warp<32, 32, VEC>(d, N, n, s);
-    case 2048: return launch_fixed_cta<2, VEC>(d, N, n, s);
-    case 4096: return launch_fixed_cta<4, VEC>(d, N, n, s);
+    case 2048: return launch_fixed_cta<2, 2, VEC>(d, N, n, s);
+    case 4096:  // 3 real warps suffice up to 3072 (the 4th block is all padding)
+      return n <= 3072 ? launch_fixed_cta<4, 3, VEC>(d, N, n, s) : launch_fixed_cta<4, 4, VEC>(d, N, n, s);
   }
   return cudaErrorInvalidValue;
 }
@@ -118,11 +119,11 @@ cudaError_t launch_offsets_warp(uint32_t* d, const int64_t* off, int64_t N, cuda
   return cudaGetLastError();
 }
 
-template <int W>
+template <int W, int WR>
 cudaError_t launch_offsets_cta(uint32_t* d, const int64_t* off, int64_t N, cudaStream_t s) {
-  auto k = gas::k_offsets_cta<W>;
-  const int grid = persistent_grid(k, 32 * W, (N + 31) / 32);
-  k<<<grid, 32 * W, 0, s>>>(d, off, N, 1u);
+  auto k = gas::k_offsets_cta<W, WR>;
+  const int grid = persistent_grid(k, 32 * WR, (N + 31) / 32);
+  k<<<grid, 32 * WR, 0, s>>>(d, off, N, 1u);
   return cudaGetLastError();
 }
 
@@ -138,8 +139,9 @@ cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, i
     case 256: return launch_offsets_warp<32, 8>(d, off, N, s);
     case 512: return launch_offsets_warp<32, 16>(d, off, N, s);
     case 1024: return launch_offsets_warp<32, 32>(d, off, N, s);
-    case 2048: return launch_offsets_cta<2>(d, off, N, s);
-    case 4096: return launch_offsets_cta<4>(d, off, N, s);
+    case 2048: return launch_offsets_cta<2, 2>(d, off, N, s);
+    case 3072: return launch_offsets_cta<4, 3>(d, off, N, s);
+    case 4096: return launch_offsets_cta<4, 4>(d, off, N, s);
   }
   return cudaErrorInvalidValue;
 }
@@ -231,9 +233,12 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
     if (h) return GAS_ERROR_INVALID_VALUE;
   }
   uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
-  const int32_t top = size_class(max_array_len);
-  for (int32_t P = 2; P <= top; P <<= 1) {
-    const cudaError_t e = dispatch_offsets_class(P, d, d_offsets, num_arrays, stream);
+  // size classes: 2, 4, ..., 2048 (len in (P/2, P]), then (2048, 3072] and (3072, 4096]
+  const int32_t classes[] = {2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096};
+  const int32_t lower[] = {1, 2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072};
+  for (int c = 0; c < 13; ++c) {
+    if (lower[c] >= max_array_len) break;
+    const cudaError_t e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, stream);
     if (e != cudaSuccess) return cuda_fail(e);
     g_launches.fetch_add(1, std::memory_order_relaxed);
   }

@@ -115,7 +115,7 @@ __global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS) k_fixed_warp(
     const bool valid = a < N;
     uint32_t k[KPT];
     load_keys<KPT, G, VEC>(k, d + (valid ? a : 0) * (int64_t)n, n, g, valid);
-    if constexpr (KPT == 32 && G == 32) sort1024_warp(k, lane, reinterpret_cast<uint32_t*>(sb), one);
+    if constexpr (KPT == 32 && G >= 2) sort_group_warp<G>(k, g, reinterpret_cast<uint32_t*>(sb), one);
     else Bitonic<KPT, G, 1>::sort(k, g, 0, nullptr, one);
     stage_out_words<KPT>(k, sb, grp * P + g * KPT);
     __syncwarp();
@@ -205,17 +205,21 @@ __global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS)
   }
 }
 
-// CTA-level classes: P = 1024 * W (W = 2, 4), one array per CTA of 32W threads.
-template <int W, bool VEC>
-__global__ void __launch_bounds__(32 * W) k_fixed_cta(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
-  constexpr int KPT = 32, T = 32 * W, P = KPT * T;
-  __shared__ uint4 smem[P / 4];
+// CTA-level classes: P = 1024 * W (W = 2, 4), one array per CTA of 32*WR
+// threads (WR <= W real warps: n <= 1024 * WR, see sort_cta).
+template <int W, int WR, bool VEC>
+__global__ void __launch_bounds__(32 * WR, (16 / WR > 0 ? 16 / WR : 1)) k_fixed_cta(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+  constexpr int KPT = 32, T = 32 * WR, P = KPT * 32 * W;
+  __shared__ uint4 smem[P / 4];          // cross-warp exchange, then rank-order staging
+  __shared__ uint4 wsm[WR][256];         // per-warp transpose scratch (4 KB each)
   uint32_t* xs = reinterpret_cast<uint32_t*>(smem);
-  const int t = threadIdx.x, g = t & 31;
+  const int t = threadIdx.x, lane = t & 31;
+  uint32_t* wbuf = reinterpret_cast<uint32_t*>(wsm[t >> 5]);
   for (int64_t a = blockIdx.x; a < N; a += gridDim.x) {
     uint32_t k[KPT];
     load_keys<KPT, T, VEC>(k, d + a * (int64_t)n, n, t, true);
-    Bitonic<KPT, 32, W>::sort(k, g, t, xs, one);
+    fill_virtual<W, WR>(xs, t);
+    sort_cta<W>(k, t, lane, xs, wbuf, one);
     __syncthreads();
     stage_out_words<KPT>(k, smem, t * KPT);
     __syncthreads();
@@ -249,7 +253,7 @@ __device__ __forceinline__ bool in_class(int64_t len, int P) {
 }
 
 template <int KPT, int G>
-__global__ void __launch_bounds__(kWarpBlock) k_offsets_warp(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
+__global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS) k_offsets_warp(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
                                                           int64_t N, uint32_t one) {
   constexpr int GROUPS = 32 / G;
   constexpr int P = KPT * G;
@@ -273,7 +277,8 @@ __global__ void __launch_bounds__(kWarpBlock) k_offsets_warp(uint32_t* __restric
       // the other groups' slots of this round, for the store phase
       uint32_t k[KPT];
       load_keys<KPT, G, false>(k, d + lo, len, g, valid);
-      Bitonic<KPT, G, 1>::sort(k, g, 0, nullptr, one);
+      if constexpr (KPT == 32 && G >= 2) sort_group_warp<G>(k, g, reinterpret_cast<uint32_t*>(sb), one);
+      else Bitonic<KPT, G, 1>::sort(k, g, 0, nullptr, one);
       stage_out_words<KPT>(k, sb, grp * P + g * KPT);
       __syncwarp();
 #pragma unroll
@@ -295,18 +300,21 @@ __global__ void __launch_bounds__(kWarpBlock) k_offsets_warp(uint32_t* __restric
   }
 }
 
-template <int W>
-__global__ void __launch_bounds__(32 * W) k_offsets_cta(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
-                                                        int64_t N, uint32_t one) {
-  constexpr int KPT = 32, T = 32 * W, P = KPT * T;
+template <int W, int WR>
+__global__ void __launch_bounds__(32 * WR, (16 / WR > 0 ? 16 / WR : 1)) k_offsets_cta(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
+                                                         int64_t N, uint32_t one) {
+  constexpr int KPT = 32, T = 32 * WR, P = KPT * 32 * W;
+  constexpr int LO = 1024 * (WR - 1), HI = 1024 * WR;  // lengths handled: (LO, HI]
   __shared__ uint4 smem[P / 4];
+  __shared__ uint4 wsm[WR][256];
   uint32_t* xs = reinterpret_cast<uint32_t*>(smem);
   const int t = threadIdx.x, g = t & 31;
+  uint32_t* wbuf = reinterpret_cast<uint32_t*>(wsm[t >> 5]);
   for (int64_t win = (int64_t)blockIdx.x * 32; win < N; win += (int64_t)gridDim.x * 32) {
     const int64_t mine = win + g;
     int64_t my_lo = 0, my_len = 0;
     if (mine < N) { my_lo = off[mine]; my_len = off[mine + 1] - my_lo; }
-    uint32_t mask = __ballot_sync(0xffffffffu, mine < N && in_class(my_len, P));
+    uint32_t mask = __ballot_sync(0xffffffffu, mine < N && my_len > LO && my_len <= HI);
     while (mask) {  // identical in every warp of the CTA
       const int pos = __ffs(mask) - 1;
       mask &= mask - 1;
@@ -314,7 +322,8 @@ __global__ void __launch_bounds__(32 * W) k_offsets_cta(uint32_t* __restrict__ d
       const int len = (int)__shfl_sync(0xffffffffu, my_len, pos);
       uint32_t k[KPT];
       load_keys<KPT, T, false>(k, d + lo, len, t, true);
-      Bitonic<KPT, 32, W>::sort(k, g, t, xs, one);
+      fill_virtual<W, WR>(xs, t);
+      sort_cta<W>(k, t, g, xs, wbuf, one);
       __syncthreads();
       stage_out_words<KPT>(k, smem, t * KPT);
       __syncthreads();

@@ -117,24 +117,76 @@ __device__ __forceinline__ void shfl_cleaner(uint32_t (&k)[32], int m, bool uppe
 #endif
 constexpr int kLevelUnroll = GAS_LEVEL_UNROLL;
 
-// Sort 1024 keys held by the warp (32 per lane, layout A in and out).
-// `sm` is the warp's 1024-word shared buffer.
-__device__ __forceinline__ void sort1024_warp(uint32_t (&k)[32], int lane, uint32_t* sm, uint32_t one) {
+// Sort P = 32*G keys held by a group of G lanes (32 per lane, layout A in and
+// out; G in {2, ..., 32}, groups aligned inside the warp). Levels 6 ..
+// 5+log2(G) run in one rolled loop; for G = 32 the lane-distance cleaners of
+// levels 8-10 go through a transpose (`sm`: the warp's 1024-word buffer),
+// otherwise they are SHFL stages.
+template <int G>
+__device__ __forceinline__ void sort_group_warp(uint32_t (&k)[32], int g, uint32_t* sm, uint32_t one) {
+  constexpr int LOGG = Log2<G>::value;
   sort32_regs(k, one);
 #pragma unroll kLevelUnroll
-  for (int lk = 6; lk <= 10; ++lk) {
-    shfl_mirror(k, (1 << (lk - 5)) - 1, lane & (1 << (lk - 6)));
+  for (int lk = 6; lk <= 5 + LOGG; ++lk) {
+    shfl_mirror(k, (1 << (lk - 5)) - 1, g & (1 << (lk - 6)));
     if (lk == 7) {
-      shfl_cleaner(k, 1, lane & 1);
-    } else if (lk >= 8) {
-      transpose_ab(k, sm, lane);  // element i = r*32 + lane: lane bits became register bits
+      shfl_cleaner(k, 1, g & 1);
+    } else if (G == 32 && lk >= 8) {
+      transpose_ab(k, sm, g);  // element i = r*32 + lane: lane bits became register bits
       if (lk == 10) Bitonic<32, 1, 1>::reg_stage<8>(k, one);
       if (lk >= 9) Bitonic<32, 1, 1>::reg_stage<4>(k, one);
       Bitonic<32, 1, 1>::reg_stage<2>(k, one);
       Bitonic<32, 1, 1>::reg_stage<1>(k, one);
-      transpose_ba(k, sm, lane);
+      transpose_ba(k, sm, g);
+    } else if (lk >= 8) {
+#pragma unroll 1
+      for (int m = 1 << (lk - 7); m >= 1; m >>= 1) shfl_cleaner(k, m, g & m);
     }
     cleaners32(k, one);
+  }
+}
+
+__device__ __forceinline__ void sort1024_warp(uint32_t (&k)[32], int lane, uint32_t* sm, uint32_t one) {
+  sort_group_warp<32>(k, lane, sm, one);
+}
+
+// Sort a bitonic 1024-sequence held by the warp (layout A): the half-cleaner
+// cascade at distances 512 .. 1 (lane distances via a transpose to layout B).
+__device__ __forceinline__ void cleaners1024_warp(uint32_t (&k)[32], int lane, uint32_t* sm, uint32_t one) {
+  transpose_ab(k, sm, lane);
+  cleaners32(k, one);  // element distances 512 .. 32 are register distances 16 .. 1 in layout B
+  transpose_ba(k, sm, lane);
+  cleaners32(k, one);
+}
+
+// One array of P = 1024 * W keys owned by a CTA of W warps (t = w*32 + lane):
+// each warp sorts its 1024-block with sort1024_warp, then the merge levels
+// 11 .. log2(P) run their cross-warp stages through shared memory (`xs`, P
+// words, element (t, r) at xs[r*32W + t]) and finish inside each warp.
+// A CTA may run with fewer real warps than W (lengths <= 1024 * real warps):
+// the missing warps' blocks are all padding, their xs slots hold kPadKey
+// (fill_virtual), and since they are the highest blocks every real element
+// is the lower partner of a padding element, keeps its own value, and the
+// network result for the real elements is unchanged.
+template <int W>
+__device__ __forceinline__ void sort_cta(uint32_t (&k)[32], int t, int lane, uint32_t* xs, uint32_t* wbuf,
+                                         uint32_t one) {
+  using B = Bitonic<32, 32, W>;
+  sort1024_warp(k, lane, wbuf, one);
+#pragma unroll 1
+  for (int lk = 11; lk <= B::LOGP; ++lk) {
+    const int K = 1 << lk;
+    B::smem_stage(k, xs, t, (K - 1) >> 5, 31, t & ((K >> 1) >> 5));  // mirror, across warps
+    for (int j = K >> 2; j >= 1024; j >>= 1) B::smem_stage(k, xs, t, j >> 5, 0, t & (j >> 5));
+    cleaners1024_warp(k, lane, wbuf, one);
+  }
+}
+
+template <int W, int WR>
+__device__ __forceinline__ void fill_virtual(uint32_t* xs, int t) {
+  if constexpr (WR < W) {
+    constexpr int VT = 32 * (W - WR);  // virtual threads
+    for (int i = t; i < 32 * VT; i += 32 * WR) xs[(i / VT) * (32 * W) + 32 * WR + i % VT] = 0xFFFFFFFFu;
   }
 }
 
