@@ -264,14 +264,19 @@ gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array
   if (num_arrays == 0 || array_len <= 1) return GAS_SUCCESS;
   if (array_len > kMaxLen) return GAS_ERROR_UNSUPPORTED;
   if (h_data == nullptr || (reinterpret_cast<uintptr_t>(h_data) & 3u)) return GAS_ERROR_INVALID_VALUE;
-  constexpr int kSlots = 3;
-  constexpr int64_t kChunkBytes = 256ll << 20;
+  constexpr int kSlots = 4;
+  const char* env_chunk = std::getenv("GAS_HOST_CHUNK_MB");  // tuning knob (default 128 MB)
+  const char* env_slots = std::getenv("GAS_HOST_SLOTS");     // 2..4 (default 3)
+  const int64_t kChunkBytes = (env_chunk ? std::atoll(env_chunk) : 128ll) << 20;
+  const int want_slots = env_slots ? std::atoi(env_slots) : 3;
   const int64_t row = (int64_t)array_len * 4;
   int64_t per_chunk = kChunkBytes / row;
   if (per_chunk < 1) per_chunk = 1;
   if (per_chunk > num_arrays) per_chunk = num_arrays;
   const int64_t nchunks = (num_arrays + per_chunk - 1) / per_chunk;
-  const int slots = (int)(nchunks < kSlots ? nchunks : kSlots);
+  int slots = (int)(nchunks < want_slots ? nchunks : want_slots);
+  if (slots > kSlots) slots = kSlots;
+  if (slots < 1) slots = 1;
   cudaStream_t st[kSlots] = {};
   float* buf[kSlots] = {};
   gas_status status = GAS_SUCCESS;
