@@ -76,8 +76,9 @@ gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len,
  *                  on the device first (with a stream synchronisation) and a
  *                  violation returns GAS_ERROR_INVALID_VALUE with nothing sorted.
  *   max_array_len > gas_max_array_len(): GAS_ERROR_UNSUPPORTED.
- * One kernel launch per size class up to max_array_len (at most 13 launches:
- * powers of two up to 2048, then (2048, 3072] and (3072, 4096]).
+ * One kernel launch per size class up to max_array_len (at most 17 launches:
+ * powers of two up to 2048, then (2048,3072], (3072,4096], (4096,6144],
+ * (6144,8192], (8192,12288], (12288,16384]).
  */
 gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int64_t num_arrays,
                                    int32_t max_array_len, cudaStream_t stream);
@@ -87,7 +88,8 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
  * §8(f) row f2): keys as in gas_sort_arrays, d_values[i*n + j] is carried with
  * d_keys[i*n + j]. STABLE: equal keys (identical bit patterns) keep their input
  * order, so the payload order is unique (reading C-2). Same argument rules as
- * gas_sort_arrays; both pointers 4-byte aligned.
+ * gas_sort_arrays (both pointers 4-byte aligned), except that array_len is
+ * limited to 8192 (GAS_ERROR_UNSUPPORTED above).
  */
 gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays, int32_t array_len,
                           cudaStream_t stream);
@@ -105,7 +107,8 @@ gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays,
  */
 gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array_len);
 
-/* Largest supported array length (4096: the paper's spectra bound). */
+/* Largest supported array length of gas_sort_arrays / _offsets / _host: 16384,
+   4x the paper's spectra bound of ~4000 peaks. */
 int32_t gas_max_array_len(void);
 
 /* Static, human-readable name of a status code. */

@@ -13,7 +13,8 @@
 
 namespace {
 
-constexpr int32_t kMaxLen = 4096;  // spectra bound of P:L170-173, rounded to a size class
+constexpr int32_t kMaxPairsLen = 8192;  // 64-bit network elements: 8 KB of SMEM per 1024
+constexpr int32_t kMaxLen = 16384;  // 4x the spectra bound of P:L170-173
 
 thread_local int g_last_cuda_error = 0;
 std::atomic<int64_t> g_launches{0};
@@ -56,12 +57,36 @@ cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   return cudaGetLastError();
 }
 
+template <typename K>
+int persistent_grid_smem(K kernel, int threads, int smem, int64_t blocks_needed) {
+  int per_sm = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kernel, threads, smem) != cudaSuccess || per_sm <= 0)
+    per_sm = 1;
+  const int64_t cap = (int64_t)per_sm * num_sms();
+  return (int)(blocks_needed < cap ? (blocks_needed > 0 ? blocks_needed : 1) : cap);
+}
+
 template <int W, int WR, bool VEC>
 cudaError_t launch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   auto k = gas::k_fixed_cta<W, WR, VEC>;
-  const int grid = persistent_grid(k, 32 * WR, N);
-  k<<<grid, 32 * WR, 0, s>>>(d, N, n, 1u);
+  constexpr int smem = gas::cta_smem_bytes<W, WR>();
+  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  if (e != cudaSuccess) return e;
+  k<<<persistent_grid_smem(k, 32 * WR, smem, N), 32 * WR, smem, s>>>(d, N, n, 1u);
   return cudaGetLastError();
+}
+
+// Fixed-length CTA classes (n > 1024): W warps' network, WR = ceil(n / 1024) real
+// warps rounded to the instantiated set (padding blocks are virtual, see sort_cta).
+template <bool VEC>
+cudaError_t dispatch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  if (n <= 2048) return launch_fixed_cta<2, 2, VEC>(d, N, n, s);
+  if (n <= 3072) return launch_fixed_cta<4, 3, VEC>(d, N, n, s);
+  if (n <= 4096) return launch_fixed_cta<4, 4, VEC>(d, N, n, s);
+  if (n <= 6144) return launch_fixed_cta<8, 6, VEC>(d, N, n, s);
+  if (n <= 8192) return launch_fixed_cta<8, 8, VEC>(d, N, n, s);
+  if (n <= 12288) return launch_fixed_cta<16, 12, VEC>(d, N, n, s);
+  return launch_fixed_cta<16, 16, VEC>(d, N, n, s);
 }
 
 bool env_flag(const char* name) {
@@ -103,9 +128,7 @@ cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
       // the kernel is ALU/issue-bound, not latency-bound.
       if (VEC && env_flag("GAS_TMA")) return launch_fixed_1024_tma(d, N, n, s);
       return launch_fixed_warp<32, 32, VEC>(d, N, n, s);
-    case 2048: return launch_fixed_cta<2, 2, VEC>(d, N, n, s);
-    case 4096:  // 3 real warps suffice up to 3072 (the 4th block is all padding)
-      return n <= 3072 ? launch_fixed_cta<4, 3, VEC>(d, N, n, s) : launch_fixed_cta<4, 4, VEC>(d, N, n, s);
+    default: return dispatch_fixed_cta<VEC>(d, N, n, s);
   }
   return cudaErrorInvalidValue;
 }
@@ -120,10 +143,12 @@ cudaError_t launch_offsets_warp(uint32_t* d, const int64_t* off, int64_t N, cuda
 }
 
 template <int W, int WR>
-cudaError_t launch_offsets_cta(uint32_t* d, const int64_t* off, int64_t N, cudaStream_t s) {
+cudaError_t launch_offsets_cta(uint32_t* d, const int64_t* off, int64_t N, int64_t lo, int64_t hi, cudaStream_t s) {
   auto k = gas::k_offsets_cta<W, WR>;
-  const int grid = persistent_grid(k, 32 * WR, (N + 31) / 32);
-  k<<<grid, 32 * WR, 0, s>>>(d, off, N, 1u);
+  constexpr int smem = gas::cta_smem_bytes<W, WR>();
+  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  if (e != cudaSuccess) return e;
+  k<<<persistent_grid_smem(k, 32 * WR, smem, (N + 31) / 32), 32 * WR, smem, s>>>(d, off, N, lo, hi, 1u);
   return cudaGetLastError();
 }
 
@@ -139,9 +164,13 @@ cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, i
     case 256: return launch_offsets_warp<32, 8>(d, off, N, s);
     case 512: return launch_offsets_warp<32, 16>(d, off, N, s);
     case 1024: return launch_offsets_warp<32, 32>(d, off, N, s);
-    case 2048: return launch_offsets_cta<2, 2>(d, off, N, s);
-    case 3072: return launch_offsets_cta<4, 3>(d, off, N, s);
-    case 4096: return launch_offsets_cta<4, 4>(d, off, N, s);
+    case 2048: return launch_offsets_cta<2, 2>(d, off, N, 1024, 2048, s);
+    case 3072: return launch_offsets_cta<4, 3>(d, off, N, 2048, 3072, s);
+    case 4096: return launch_offsets_cta<4, 4>(d, off, N, 3072, 4096, s);
+    case 6144: return launch_offsets_cta<8, 6>(d, off, N, 4096, 6144, s);
+    case 8192: return launch_offsets_cta<8, 8>(d, off, N, 6144, 8192, s);
+    case 12288: return launch_offsets_cta<16, 12>(d, off, N, 8192, 12288, s);
+    case 16384: return launch_offsets_cta<16, 16>(d, off, N, 12288, 16384, s);
   }
   return cudaErrorInvalidValue;
 }
@@ -175,6 +204,7 @@ cudaError_t dispatch_pairs(uint32_t* k, uint32_t* v, int64_t N, int n, cudaStrea
     case 1024: return launch_pairs<32, 32, 1>(k, v, N, n, s);
     case 2048: return launch_pairs<32, 32, 2>(k, v, N, n, s);
     case 4096: return launch_pairs<32, 32, 4>(k, v, N, n, s);
+    case 8192: return launch_pairs<32, 32, 8>(k, v, N, n, s);
   }
   return cudaErrorInvalidValue;
 }
@@ -234,9 +264,9 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
   }
   uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
   // size classes: 2, 4, ..., 2048 (len in (P/2, P]), then (2048, 3072] and (3072, 4096]
-  const int32_t classes[] = {2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096};
-  const int32_t lower[] = {1, 2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072};
-  for (int c = 0; c < 13; ++c) {
+  const int32_t classes[] = {2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288, 16384};
+  const int32_t lower[] = {1, 2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288};
+  for (int c = 0; c < 17; ++c) {
     if (lower[c] >= max_array_len) break;
     const cudaError_t e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, stream);
     if (e != cudaSuccess) return cuda_fail(e);
@@ -249,7 +279,7 @@ gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays,
                           cudaStream_t stream) {
   if (num_arrays < 0 || array_len < 0) return GAS_ERROR_INVALID_VALUE;
   if (num_arrays == 0 || array_len <= 1) return GAS_SUCCESS;
-  if (array_len > kMaxLen) return GAS_ERROR_UNSUPPORTED;
+  if (array_len > kMaxPairsLen) return GAS_ERROR_UNSUPPORTED;
   if (d_keys == nullptr || d_values == nullptr || (reinterpret_cast<uintptr_t>(d_keys) & 3u) ||
       (reinterpret_cast<uintptr_t>(d_values) & 3u))
     return GAS_ERROR_INVALID_VALUE;

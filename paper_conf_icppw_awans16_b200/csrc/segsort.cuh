@@ -205,16 +205,21 @@ __global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS)
   }
 }
 
-// CTA-level classes: P = 1024 * W (W = 2, 4), one array per CTA of 32*WR
+template <int W, int WR>
+constexpr int cta_smem_bytes() { return 1024 * W * 4 + WR * 4096; }
+
+// CTA-level classes: P = 1024 * W (W = 2, 4, 8, 16), one array per CTA of 32*WR
 // threads (WR <= W real warps: n <= 1024 * WR, see sort_cta).
 template <int W, int WR, bool VEC>
 __global__ void __launch_bounds__(32 * WR, (16 / WR > 0 ? 16 / WR : 1)) k_fixed_cta(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   constexpr int KPT = 32, T = 32 * WR, P = KPT * 32 * W;
-  __shared__ uint4 smem[P / 4];          // cross-warp exchange, then rank-order staging
-  __shared__ uint4 wsm[WR][256];         // per-warp transpose scratch (4 KB each)
+  // dynamic shared memory (cta_smem_bytes<W, WR>()): P words of cross-warp
+  // exchange / rank-order staging, then a 4 KB transpose scratch per warp
+  extern __shared__ __align__(16) uint4 cta_smem[];
+  uint4* smem = cta_smem;
   uint32_t* xs = reinterpret_cast<uint32_t*>(smem);
   const int t = threadIdx.x, lane = t & 31;
-  uint32_t* wbuf = reinterpret_cast<uint32_t*>(wsm[t >> 5]);
+  uint32_t* wbuf = reinterpret_cast<uint32_t*>(cta_smem + P / 4 + (t >> 5) * 256);
   for (int64_t a = blockIdx.x; a < N; a += gridDim.x) {
     uint32_t k[KPT];
     load_keys<KPT, T, VEC>(k, d + a * (int64_t)n, n, t, true);
@@ -302,14 +307,14 @@ __global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS) k_offsets_war
 
 template <int W, int WR>
 __global__ void __launch_bounds__(32 * WR, (16 / WR > 0 ? 16 / WR : 1)) k_offsets_cta(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
-                                                         int64_t N, uint32_t one) {
+                                                         int64_t N, int64_t LO, int64_t HI, uint32_t one) {
+  // handles the arrays with LO < length <= HI (HI <= 1024 * WR)
   constexpr int KPT = 32, T = 32 * WR, P = KPT * 32 * W;
-  constexpr int LO = 1024 * (WR - 1), HI = 1024 * WR;  // lengths handled: (LO, HI]
-  __shared__ uint4 smem[P / 4];
-  __shared__ uint4 wsm[WR][256];
+  extern __shared__ __align__(16) uint4 cta_smem[];
+  uint4* smem = cta_smem;
   uint32_t* xs = reinterpret_cast<uint32_t*>(smem);
   const int t = threadIdx.x, g = t & 31;
-  uint32_t* wbuf = reinterpret_cast<uint32_t*>(wsm[t >> 5]);
+  uint32_t* wbuf = reinterpret_cast<uint32_t*>(cta_smem + P / 4 + (t >> 5) * 256);
   for (int64_t win = (int64_t)blockIdx.x * 32; win < N; win += (int64_t)gridDim.x * 32) {
     const int64_t mine = win + g;
     int64_t my_lo = 0, my_len = 0;

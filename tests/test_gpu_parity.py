@@ -55,7 +55,8 @@ def oracle_sorted(host: np.ndarray) -> np.ndarray:
 
 
 SIZES = [2, 3, 4, 5, 7, 8, 9, 15, 16, 17, 31, 32, 33, 63, 64, 65, 100, 127, 128, 129, 255, 256, 257,
-         500, 511, 512, 513, 999, 1000, 1023, 1024, 1025, 1500, 2047, 2048, 2049, 3000, 4000, 4095, 4096]
+         500, 511, 512, 513, 999, 1000, 1023, 1024, 1025, 1500, 2047, 2048, 2049, 3000, 3072, 3073, 4000, 4095,
+         4096, 4097, 5000, 6144, 6145, 8192, 8193, 12288, 12289, 16383, 16384]
 
 
 @pytest.mark.parametrize("n", SIZES)
@@ -150,6 +151,7 @@ def gpu_sort_offsets(data: np.ndarray, off: np.ndarray, lead: int = 3, max_len: 
 def test_offsets_all_classes(dist):
     lens = datagen.lengths(201, 0, 3000, 0, 4096)
     lens[:12] = [0, 1, 2, 3, 4096, 0, 5, 4095, 1, 2049, 33, 1024]
+    lens[12:24] = [3072, 3073, 6144, 6145, 8192, 8193, 12288, 12289, 16384, 4097, 16383, 5000]
     off = datagen.offsets_from_lengths(lens)
     data = datagen.ragged(dist, 201, 0, off)
     expect = data.copy()
@@ -288,7 +290,7 @@ def test_config1_full_size_sampled(dist):
 # ------------------------------------------------------------ stable pairs (f2)
 
 
-@pytest.mark.parametrize("n", [2, 3, 16, 33, 100, 512, 1000, 1024, 1500, 2048, 4000, 4096])
+@pytest.mark.parametrize("n", [2, 3, 16, 33, 100, 512, 1000, 1024, 1500, 2048, 4000, 4096, 6000, 8192])
 @pytest.mark.parametrize("dist", ["dup16", "special_mix", "uniform_bits"])
 def test_pairs_stable_vs_oracle(n, dist):
     N = max(3, min(200, 100000 // n))
