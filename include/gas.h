@@ -19,8 +19,9 @@
  *
  * Conventions for every entry point:
  *   - Pointers named d_* are DEVICE memory of the current device, owned by
- *     the caller; the library never allocates on the device-resident entry
- *     points (zero workspace) and never calls cudaSetDevice.
+ *     the caller; gas_sort_arrays and gas_sort_pairs allocate nothing (zero
+ *     workspace); the offsets variant uses 56 bytes (see there); the library
+ *     never calls cudaSetDevice.
  *   - Work is enqueued on `stream` (0 = legacy default stream) and the call
  *     returns without a host synchronisation. Argument and launch-
  *     configuration errors are returned synchronously; faults during
@@ -76,6 +77,8 @@ gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len,
  *                  on the device first (with a stream synchronisation) and a
  *                  violation returns GAS_ERROR_INVALID_VALUE with nothing sorted.
  *   max_array_len > gas_max_array_len(): GAS_ERROR_UNSUPPORTED.
+ * Workspace: 56 bytes of stream-ordered device memory (cudaMallocAsync /
+ * cudaFreeAsync on `stream`) for dynamic scheduling when max_array_len > 1024.
  * One kernel launch per size class up to max_array_len (at most 17 launches:
  * powers of two up to 2048, then (2048,3072], (3072,4096], (4096,6144],
  * (6144,8192], (8192,12288], (12288,16384]).

@@ -143,16 +143,18 @@ cudaError_t launch_offsets_warp(uint32_t* d, const int64_t* off, int64_t N, cuda
 }
 
 template <int W, int WR>
-cudaError_t launch_offsets_cta(uint32_t* d, const int64_t* off, int64_t N, int64_t lo, int64_t hi, cudaStream_t s) {
+cudaError_t launch_offsets_cta(uint32_t* d, const int64_t* off, int64_t N, int64_t lo, int64_t hi,
+                               unsigned long long* ctr, cudaStream_t s) {
   auto k = gas::k_offsets_cta<W, WR>;
   constexpr int smem = gas::cta_smem_bytes<W, WR>();
   const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
   if (e != cudaSuccess) return e;
-  k<<<persistent_grid_smem(k, 32 * WR, smem, (N + 31) / 32), 32 * WR, smem, s>>>(d, off, N, lo, hi, 1u);
+  k<<<persistent_grid_smem(k, 32 * WR, smem, (N + 31) / 32), 32 * WR, smem, s>>>(d, off, N, lo, hi, ctr, 1u);
   return cudaGetLastError();
 }
 
-cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, int64_t N, cudaStream_t s) {
+cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, int64_t N, unsigned long long* ctr,
+                                   cudaStream_t s) {
   switch (P) {
     case 2: return launch_offsets_warp<2, 1>(d, off, N, s);
     case 4: return launch_offsets_warp<4, 1>(d, off, N, s);
@@ -164,13 +166,13 @@ cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, i
     case 256: return launch_offsets_warp<32, 8>(d, off, N, s);
     case 512: return launch_offsets_warp<32, 16>(d, off, N, s);
     case 1024: return launch_offsets_warp<32, 32>(d, off, N, s);
-    case 2048: return launch_offsets_cta<2, 2>(d, off, N, 1024, 2048, s);
-    case 3072: return launch_offsets_cta<4, 3>(d, off, N, 2048, 3072, s);
-    case 4096: return launch_offsets_cta<4, 4>(d, off, N, 3072, 4096, s);
-    case 6144: return launch_offsets_cta<8, 6>(d, off, N, 4096, 6144, s);
-    case 8192: return launch_offsets_cta<8, 8>(d, off, N, 6144, 8192, s);
-    case 12288: return launch_offsets_cta<16, 12>(d, off, N, 8192, 12288, s);
-    case 16384: return launch_offsets_cta<16, 16>(d, off, N, 12288, 16384, s);
+    case 2048: return launch_offsets_cta<2, 2>(d, off, N, 1024, 2048, ctr, s);
+    case 3072: return launch_offsets_cta<4, 3>(d, off, N, 2048, 3072, ctr + 1, s);
+    case 4096: return launch_offsets_cta<4, 4>(d, off, N, 3072, 4096, ctr + 2, s);
+    case 6144: return launch_offsets_cta<8, 6>(d, off, N, 4096, 6144, ctr + 3, s);
+    case 8192: return launch_offsets_cta<8, 8>(d, off, N, 6144, 8192, ctr + 4, s);
+    case 12288: return launch_offsets_cta<16, 12>(d, off, N, 8192, 12288, ctr + 5, s);
+    case 16384: return launch_offsets_cta<16, 16>(d, off, N, 12288, 16384, ctr + 6, s);
   }
   return cudaErrorInvalidValue;
 }
@@ -263,14 +265,28 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
     if (h) return GAS_ERROR_INVALID_VALUE;
   }
   uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
+  // 7 window counters for the CTA classes' dynamic scheduling (stream-ordered, 56 bytes)
+  unsigned long long* ctr = nullptr;
+  if (max_array_len > 1024) {
+    cudaError_t e = cudaMallocAsync(&ctr, 7 * sizeof(unsigned long long), stream);
+    if (e == cudaSuccess) e = cudaMemsetAsync(ctr, 0, 7 * sizeof(unsigned long long), stream);
+    if (e != cudaSuccess) return cuda_fail(e);
+  }
   // size classes: 2, 4, ..., 2048 (len in (P/2, P]), then (2048, 3072] and (3072, 4096]
   const int32_t classes[] = {2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288, 16384};
   const int32_t lower[] = {1, 2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288};
   for (int c = 0; c < 17; ++c) {
     if (lower[c] >= max_array_len) break;
-    const cudaError_t e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, stream);
-    if (e != cudaSuccess) return cuda_fail(e);
+    const cudaError_t e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, ctr, stream);
+    if (e != cudaSuccess) {
+      if (ctr) cudaFreeAsync(ctr, stream);
+      return cuda_fail(e);
+    }
     g_launches.fetch_add(1, std::memory_order_relaxed);
+  }
+  if (ctr) {
+    const cudaError_t e = cudaFreeAsync(ctr, stream);
+    if (e != cudaSuccess) return cuda_fail(e);
   }
   return GAS_SUCCESS;
 }

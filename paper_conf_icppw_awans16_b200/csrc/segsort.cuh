@@ -307,7 +307,8 @@ __global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS) k_offsets_war
 
 template <int W, int WR>
 __global__ void __launch_bounds__(32 * WR, (16 / WR > 0 ? 16 / WR : 1)) k_offsets_cta(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
-                                                         int64_t N, int64_t LO, int64_t HI, uint32_t one) {
+                                                         int64_t N, int64_t LO, int64_t HI,
+                                                         unsigned long long* __restrict__ ctr, uint32_t one) {
   // handles the arrays with LO < length <= HI (HI <= 1024 * WR)
   constexpr int KPT = 32, T = 32 * WR, P = KPT * 32 * W;
   extern __shared__ __align__(16) uint4 cta_smem[];
@@ -315,7 +316,18 @@ __global__ void __launch_bounds__(32 * WR, (16 / WR > 0 ? 16 / WR : 1)) k_offset
   uint32_t* xs = reinterpret_cast<uint32_t*>(smem);
   const int t = threadIdx.x, g = t & 31;
   uint32_t* wbuf = reinterpret_cast<uint32_t*>(cta_smem + P / 4 + (t >> 5) * 256);
-  for (int64_t win = (int64_t)blockIdx.x * 32; win < N; win += (int64_t)gridDim.x * 32) {
+  // windows of 32 arrays are handed out dynamically through `ctr` (one counter
+  // per launch, zeroed by the host) so that CTAs finish together even though
+  // the number of in-class arrays per window varies
+  __shared__ int64_t s_win;
+  auto next_window = [&]() -> int64_t {
+    if (t == 0) s_win = (int64_t)atomicAdd(ctr, 1ull) * 32;
+    __syncthreads();
+    const int64_t w = s_win;
+    __syncthreads();
+    return w;
+  };
+  for (int64_t win = next_window(); win < N; win = next_window()) {
     const int64_t mine = win + g;
     int64_t my_lo = 0, my_len = 0;
     if (mine < N) { my_lo = off[mine]; my_len = off[mine + 1] - my_lo; }
