@@ -123,27 +123,38 @@ constexpr int kLevelUnroll = GAS_LEVEL_UNROLL;
 // levels 8-10 go through a transpose (`sm`: the warp's 1024-word buffer),
 // otherwise they are SHFL stages.
 template <int G>
+__device__ __forceinline__ void level_step(uint32_t (&k)[32], int g, uint32_t* sm, uint32_t one, int lk) {
+  shfl_mirror(k, (1 << (lk - 5)) - 1, g & (1 << (lk - 6)));
+  if (lk == 7) {
+    shfl_cleaner(k, 1, g & 1);
+  } else if (G == 32 && lk >= 8) {
+    transpose_ab(k, sm, g);  // element i = r*32 + lane: lane bits became register bits
+    if (lk == 10) Bitonic<32, 1, 1>::reg_stage<8>(k, one);
+    if (lk >= 9) Bitonic<32, 1, 1>::reg_stage<4>(k, one);
+    Bitonic<32, 1, 1>::reg_stage<2>(k, one);
+    Bitonic<32, 1, 1>::reg_stage<1>(k, one);
+    transpose_ba(k, sm, g);
+  } else if (lk >= 8) {
+#pragma unroll 1
+    for (int m = 1 << (lk - 7); m >= 1; m >>= 1) shfl_cleaner(k, m, g & m);
+  }
+  cleaners32(k, one);
+}
+
+#ifndef GAS_UNROLLED_LOW_LEVELS
+#define GAS_UNROLLED_LOW_LEVELS 0  // levels 6..5+this are unrolled, the rest rolled
+#endif
+
+template <int G>
 __device__ __forceinline__ void sort_group_warp(uint32_t (&k)[32], int g, uint32_t* sm, uint32_t one) {
   constexpr int LOGG = Log2<G>::value;
+  constexpr int TOP = 5 + LOGG;
+  constexpr int UNR = GAS_UNROLLED_LOW_LEVELS < LOGG ? GAS_UNROLLED_LOW_LEVELS : LOGG;
   sort32_regs(k, one);
+#pragma unroll
+  for (int lk = 6; lk < 6 + UNR; ++lk) level_step<G>(k, g, sm, one, lk);
 #pragma unroll kLevelUnroll
-  for (int lk = 6; lk <= 5 + LOGG; ++lk) {
-    shfl_mirror(k, (1 << (lk - 5)) - 1, g & (1 << (lk - 6)));
-    if (lk == 7) {
-      shfl_cleaner(k, 1, g & 1);
-    } else if (G == 32 && lk >= 8) {
-      transpose_ab(k, sm, g);  // element i = r*32 + lane: lane bits became register bits
-      if (lk == 10) Bitonic<32, 1, 1>::reg_stage<8>(k, one);
-      if (lk >= 9) Bitonic<32, 1, 1>::reg_stage<4>(k, one);
-      Bitonic<32, 1, 1>::reg_stage<2>(k, one);
-      Bitonic<32, 1, 1>::reg_stage<1>(k, one);
-      transpose_ba(k, sm, g);
-    } else if (lk >= 8) {
-#pragma unroll 1
-      for (int m = 1 << (lk - 7); m >= 1; m >>= 1) shfl_cleaner(k, m, g & m);
-    }
-    cleaners32(k, one);
-  }
+  for (int lk = 6 + UNR; lk <= TOP; ++lk) level_step<G>(k, g, sm, one, lk);
 }
 
 __device__ __forceinline__ void sort1024_warp(uint32_t (&k)[32], int lane, uint32_t* sm, uint32_t one) {
