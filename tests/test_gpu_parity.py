@@ -317,3 +317,22 @@ def test_pairs_payload_is_original_position():
         np.testing.assert_array_equal(keys[i][v[i]], k[i])
         for kv in np.unique(k[i]):
             assert np.all(np.diff(v[i][k[i] == kv].astype(np.int64)) > 0)
+
+
+def test_config2_ten_million_arrays_64bit_indexing():
+    """BASELINE.json configs[2] per-GPU size: 10^7 x 1000 = 10^10 elements (> 2^31,
+    so every element offset must be 64-bit). Sampled rows on both sides of the
+    2^31-element boundary, bit-exact vs the oracle; all rows sorted."""
+    N, n = 10_000_000, 1000
+    seed = datagen.config_seed(2)
+    x = torch.empty(N, n, dtype=torch.float32, device=DEV)
+    datagen.fixed_device(x, "paper_uniform", seed, 0, N, n)
+    gas.gas_sort_arrays(x)
+    torch.cuda.synchronize()
+    assert _row_keys_sorted(x)
+    boundary = (2**31) // n
+    rows = np.unique(np.concatenate([np.arange(boundary - 3, boundary + 4), [0, N - 1],
+                                     np.random.default_rng(3).choice(N, 500, replace=False)]))
+    expect = oracle_sorted(datagen.rows("paper_uniform", seed, rows, n))
+    got = x[torch.from_numpy(rows).to(DEV)].view(torch.int32).cpu().numpy().view(np.uint32)
+    np.testing.assert_array_equal(got, expect)
