@@ -51,6 +51,8 @@ def parse():
     p.add_argument("--no-e2e", action="store_true")
     p.add_argument("--no-cpu-baseline", action="store_true")
     p.add_argument("--e2e-steps", type=int, default=3)
+    p.add_argument("--dist-backend", default="nccl", choices=["nccl", "gloo"],
+                   help="process-group backend under torchrun (gloo: several ranks may share one GPU, for testing)")
     p.add_argument("--cpu-seconds", type=float, default=10.0, help="target CPU time of the oracle sample")
     return p.parse_args()
 
@@ -241,13 +243,21 @@ def main():
     import paper_conf_icppw_awans16_b200 as gas
 
     rank, world, local = dist_env()
+    if local >= torch.cuda.device_count():
+        if args.dist_backend != "gloo":
+            raise SystemExit(f"LOCAL_RANK {local} but only {torch.cuda.device_count()} GPUs")
+        local %= torch.cuda.device_count()  # testing mode: several gloo ranks share a GPU
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
     pg = None
-    if world > 1:
+    if "RANK" in os.environ and "WORLD_SIZE" in os.environ:  # launched by torchrun (any world size)
         import torch.distributed as dist_
-        dist_.init_process_group("nccl", device_id=dev)
+        if args.dist_backend == "nccl":
+            dist_.init_process_group("nccl", device_id=dev)
+        else:
+            dist_.init_process_group("gloo")
         pg = dist_
+    red_dev = dev if args.dist_backend == "nccl" else None  # gloo reduces host tensors
 
     def barrier():
         if pg:
@@ -306,7 +316,7 @@ def main():
     barrier()
     launches = gas.launch_count() - launches0
     per_step = [a.elapsed_time(b) for a, b in evs]
-    t_sum = shard.max_over_ranks(sum(per_step), dev)  # the slowest rank defines the job
+    t_sum = shard.max_over_ranks(sum(per_step), red_dev)  # the slowest rank defines the job
     ms_per_step = t_sum / args.steps
     total_arrays = N_rank * world
     value = total_arrays / (ms_per_step * 1e-3)
@@ -334,7 +344,7 @@ def main():
             dt = time.perf_counter() - t0
             if s > 0:
                 ts.append(dt)
-        dt = shard.max_over_ranks(sum(ts), dev) / len(ts)
+        dt = shard.max_over_ranks(sum(ts), red_dev) / len(ts)
         nbytes = N_rank * cfg["n"] * 4
         e2e = {"value": total_arrays / dt, "unit": "arrays/s", "h2d_bytes_per_step": nbytes,
                "d2h_bytes_per_step": nbytes, "ms_per_step": dt * 1e3,
@@ -354,8 +364,9 @@ def main():
             "vs_baseline": None, "dtype": "u32 (float32 bit patterns as IEEE totalOrder keys)",
             "data": "synthetic",
             "config": {"workload": cfg["name"], "num_arrays_per_gpu": N_rank, "array_len": n_desc, "dist": dist,
-                       "seed": seed, "l2": "inputs (>= 8 GB) larger than the 126 MB L2; restored from a pristine "
-                                            "copy (untimed) before every step",
+                       "seed": seed, "l2": f"inputs ({pristine.numel() * 4 / 1e9:.2f} GB per GPU) "
+                                  + ("larger than" if pristine.numel() * 4 > 126e6 else "SMALLER than (L2-resident)")
+                                  + " the 126 MB L2; restored from a pristine copy (untimed) before every step",
                        "parallelism": f"array-index shards x{world}, no collective"},
             "gbs_per_gpu": achieved_gbs,
             "roofline": {"bound": "hbm", "achieved": achieved_gbs, "peak": peak, "unit": "GB/s",
@@ -368,6 +379,7 @@ def main():
         }
         print(json.dumps(line), flush=True)
     if pg:
+        pg.barrier()
         pg.destroy_process_group()
 
 
