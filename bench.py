@@ -66,6 +66,28 @@ def measured_peak_hbm():
         return 6650.0, "fallback (B200_PROFILING.md)"
 
 
+def ncu_entry(kernel_hint: str):
+    try:
+        with open(os.path.join(ROOT, "profiles", "ncu_summary.json")) as f:
+            return json.load(f).get(kernel_hint) or {}
+    except Exception:
+        return {}
+
+
+def issue_roofline(kernel_hint: str, units_per_s: float, sm_mhz, n_sms: int):
+    """Instruction-issue view of the same kernel (the binding resource):
+    warp-instructions per array from the committed ncu capture x arrays/s, against
+    4 warp-instructions/clk/SM x SMs x the SM clock sampled during the run."""
+    e = ncu_entry(kernel_hint)
+    if not e.get("warp_instructions_per_launch") or not sm_mhz:
+        return None
+    per_unit = e["warp_instructions_per_launch"] / e["arrays_per_launch"]
+    achieved = per_unit * units_per_s
+    peak = 4 * n_sms * sm_mhz * 1e6
+    return {"bound": "issue", "achieved": achieved, "peak": peak, "unit": "warp-instr/s", "frac": achieved / peak,
+            "warp_instr_per_array": per_unit, "source": "profiles/ncu_summary.json (ncu smsp__inst_executed.sum)"}
+
+
 def ncu_traffic(kernel_hint: str):
     """Per-launch DRAM traffic of the dominant kernel from the committed ncu summary."""
     path = os.path.join(ROOT, "profiles", "ncu_summary.json")
@@ -373,6 +395,9 @@ def main():
                          "frac": achieved_gbs / peak, "traffic": ncu_traffic(kernel_hint),
                          "peak_source": peak_src, "kernel": kernel_hint,
                          "algorithmic_bytes_per_launch": alg_bytes},
+            "issue_roofline": (issue_roofline(kernel_hint, value / world, clk.summary()["sm_mhz"],
+                                              torch.cuda.get_device_properties(dev).multi_processor_count)
+                               if not ragged and cfg["n"] == 1000 else None),
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches,
             "clocks": clk.summary(), "wall_ms_timed_loop": t_wall * 1e3, "per_step_ms": per_step,
             "self_check_sorted": ok,
