@@ -24,9 +24,12 @@
 
 namespace gas {
 
-constexpr int kWarpBlock = 256;  // threads per block for the warp-level classes
+#ifndef GAS_WARP_BLOCK
+#define GAS_WARP_BLOCK 256
+#endif
+constexpr int kWarpBlock = GAS_WARP_BLOCK;  // threads per block for the warp-level classes
 #ifndef GAS_WARP_MIN_BLOCKS
-#define GAS_WARP_MIN_BLOCKS 2     // 2 x 256 threads = 16 warps/SM -> up to 128 registers (no spills)
+#define GAS_WARP_MIN_BLOCKS (512 / GAS_WARP_BLOCK)  // 16 warps/SM -> up to 128 registers (no spills)
 #endif
 
 // XOR swizzle of 16-byte chunks inside 128-byte rows: chunk c of a rank-order
