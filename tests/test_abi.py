@@ -88,3 +88,31 @@ def test_product_package_does_not_import_oracle():
             if f.endswith((".py", ".cu", ".cuh", ".h", ".cpp")):
                 src = open(os.path.join(dirpath, f)).read()
                 assert "oracle" not in re.sub(r"#.*|//.*", "", src).lower() or f.endswith(".md"), f
+
+
+def _build_c_client(tmp_path):
+    import subprocess
+    exe = str(tmp_path / "abi_check")
+    subprocess.check_call(["gcc", "-std=c11", "-Wall", "-Werror", "-I", os.path.join(ROOT, "include"),
+                           "-I", "/usr/local/cuda/include", os.path.join(ROOT, "tests", "c", "abi_check.c"),
+                           "-o", exe, "-L", os.path.dirname(gas.LIB_PATH), "-l:libgas.so",
+                           "-Wl,-rpath," + os.path.dirname(gas.LIB_PATH)])
+    return exe
+
+
+def test_plain_c_client_links_and_validates(tmp_path):
+    """include/gas.h is a C header and libgas.so is callable from C (no torch)."""
+    import subprocess
+    out = subprocess.run([_build_c_client(tmp_path)], capture_output=True, text=True)
+    assert out.returncode == 0, out.stderr
+    assert "abi_check OK" in out.stdout
+
+
+@pytest.mark.gpu
+def test_plain_c_client_sorts_through_host_entry_point(tmp_path):
+    import subprocess
+    torch = pytest.importorskip("torch")
+    if not torch.cuda.is_available():
+        pytest.skip("needs a GPU")
+    out = subprocess.run([_build_c_client(tmp_path), "gpu"], capture_output=True, text=True)
+    assert out.returncode == 0, out.stderr
