@@ -274,6 +274,7 @@ def main():
     pg = None
     if "RANK" in os.environ and "WORLD_SIZE" in os.environ:  # launched by torchrun (any world size)
         import torch.distributed as dist_
+        os.environ.setdefault("NCCL_DEBUG", "WARN")  # keep stdout to the one JSON line
         if args.dist_backend == "nccl":
             dist_.init_process_group("nccl", device_id=dev)
         else:
