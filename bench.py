@@ -274,11 +274,18 @@ def main():
     pg = None
     if "RANK" in os.environ and "WORLD_SIZE" in os.environ:  # launched by torchrun (any world size)
         import torch.distributed as dist_
-        os.environ.setdefault("NCCL_DEBUG", "WARN")  # keep stdout to the one JSON line
-        if args.dist_backend == "nccl":
-            dist_.init_process_group("nccl", device_id=dev)
-        else:
-            dist_.init_process_group("gloo")
+        saved_stdout = os.dup(1)  # NCCL prints its version banner on stdout: keep stdout to the one JSON line
+        os.dup2(2, 1)
+        try:
+            if args.dist_backend == "nccl":
+                dist_.init_process_group("nccl", device_id=dev)
+            else:
+                dist_.init_process_group("gloo")
+            dist_.barrier()
+        finally:
+            sys.stdout.flush()
+            os.dup2(saved_stdout, 1)
+            os.close(saved_stdout)
         pg = dist_
     red_dev = dev if args.dist_backend == "nccl" else None  # gloo reduces host tensors
 

@@ -113,8 +113,15 @@ struct Bitonic {
 #pragma unroll
     for (int r = 0; r < KPT; ++r) xs[r * NT + t] = k[r];
     __syncthreads();
+    // tmask >= 32: the partner is in another warp and `upper` is a warp bit, so
+    // this branch is warp-uniform and each key costs one min or one max
+    if (upper) {
 #pragma unroll
-    for (int r = 0; r < KPT; ++r) k[r] = keep(k[r], xs[(r ^ rmask) * NT + (t ^ tmask)], upper);
+      for (int r = 0; r < KPT; ++r) k[r] = max(k[r], xs[(r ^ rmask) * NT + (t ^ tmask)]);
+    } else {
+#pragma unroll
+      for (int r = 0; r < KPT; ++r) k[r] = min(k[r], xs[(r ^ rmask) * NT + (t ^ tmask)]);
+    }
   }
 
   // Half-cleaner at distance 2^LJ, then the rest of the cascade down to 1.
