@@ -105,8 +105,9 @@ gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays,
  * the two copy directions and the sort overlap) and the sorted batch is
  * written back to h_data. Pinned (page-locked) host memory gives full-duplex
  * PCIe; pageable memory works but is slower. BLOCKING: returns after the
- * result is in h_data. Uses a stream-ordered device workspace of at most
- * 3 x chunk (freed before return).
+ * result is in h_data. Device staging (3 x 128 MB by default, GAS_HOST_CHUNK_MB /
+ * GAS_HOST_SLOTS) and its streams are allocated on first use per device and kept
+ * for later calls; concurrent host-path calls on one device are serialised.
  */
 gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array_len);
 

@@ -1,6 +1,7 @@
 // gas_api.cu — the C ABI of include/gas.h: argument validation, size-class
 // dispatch, launch configuration and status codes.
 #include <atomic>
+#include <mutex>
 #include <cstdint>
 #include <cstdlib>
 #include <cstring>
@@ -219,6 +220,33 @@ __global__ void k_check_offsets(const int64_t* __restrict__ off, int64_t N, int6
   }
 }
 
+// Device staging for gas_sort_arrays_host: streams and chunk buffers are created
+// on first use and kept per device (re-used by later calls; grown on demand),
+// so repeated host sorts do not pay cudaMalloc / cudaFree (which synchronises).
+constexpr int kHostSlots = 4;
+constexpr int kMaxDevices = 64;
+struct HostStaging {
+  std::mutex mu;
+  cudaStream_t st[kHostSlots] = {};
+  float* buf[kHostSlots] = {};
+  int64_t bytes = 0;
+  cudaError_t ensure(int slots, int64_t need) {
+    cudaError_t e = cudaSuccess;
+    for (int s = 0; s < kHostSlots && e == cudaSuccess; ++s)
+      if (!st[s]) e = cudaStreamCreateWithFlags(&st[s], cudaStreamNonBlocking);
+    if (e != cudaSuccess) return e;
+    if (need > bytes) {
+      for (int s = 0; s < kHostSlots; ++s)
+        if (buf[s]) { cudaFree(buf[s]); buf[s] = nullptr; }
+      bytes = need;
+    }
+    for (int s = 0; s < slots && e == cudaSuccess; ++s)
+      if (!buf[s]) e = cudaMalloc(&buf[s], bytes);
+    return e;
+  }
+};
+HostStaging g_staging[kMaxDevices];
+
 bool env_check() {
   const char* v = std::getenv("GAS_CHECK");
   return v && std::strcmp(v, "0") != 0 && v[0] != '\0';
@@ -310,45 +338,41 @@ gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array
   if (num_arrays == 0 || array_len <= 1) return GAS_SUCCESS;
   if (array_len > kMaxLen) return GAS_ERROR_UNSUPPORTED;
   if (h_data == nullptr || (reinterpret_cast<uintptr_t>(h_data) & 3u)) return GAS_ERROR_INVALID_VALUE;
-  constexpr int kSlots = 4;
   const char* env_chunk = std::getenv("GAS_HOST_CHUNK_MB");  // tuning knob (default 128 MB)
-  const char* env_slots = std::getenv("GAS_HOST_SLOTS");     // 2..4 (default 3)
-  const int64_t kChunkBytes = (env_chunk ? std::atoll(env_chunk) : 128ll) << 20;
+  const char* env_slots = std::getenv("GAS_HOST_SLOTS");     // 1..4 (default 3)
+  const int64_t chunk_bytes = (env_chunk ? std::atoll(env_chunk) : 128ll) << 20;
   const int want_slots = env_slots ? std::atoi(env_slots) : 3;
   const int64_t row = (int64_t)array_len * 4;
-  int64_t per_chunk = kChunkBytes / row;
+  int64_t per_chunk = chunk_bytes / row;
   if (per_chunk < 1) per_chunk = 1;
   if (per_chunk > num_arrays) per_chunk = num_arrays;
   const int64_t nchunks = (num_arrays + per_chunk - 1) / per_chunk;
   int slots = (int)(nchunks < want_slots ? nchunks : want_slots);
-  if (slots > kSlots) slots = kSlots;
+  if (slots > kHostSlots) slots = kHostSlots;
   if (slots < 1) slots = 1;
-  cudaStream_t st[kSlots] = {};
-  float* buf[kSlots] = {};
+  int dev = 0;
+  cudaError_t e = cudaGetDevice(&dev);
+  if (e != cudaSuccess) return cuda_fail(e);
+  if (dev < 0 || dev >= kMaxDevices) return GAS_ERROR_UNSUPPORTED;
+  HostStaging& hs = g_staging[dev];
+  std::lock_guard<std::mutex> lock(hs.mu);  // one host-path sort per device at a time (they share PCIe anyway)
+  e = hs.ensure(slots, per_chunk * row);
+  if (e != cudaSuccess) return cuda_fail(e);
   gas_status status = GAS_SUCCESS;
-  cudaError_t e = cudaSuccess;
-  for (int s = 0; s < slots && e == cudaSuccess; ++s) {
-    e = cudaStreamCreateWithFlags(&st[s], cudaStreamNonBlocking);
-    if (e == cudaSuccess) e = cudaMalloc(&buf[s], per_chunk * row);
-  }
   for (int64_t c = 0; c < nchunks && e == cudaSuccess && status == GAS_SUCCESS; ++c) {
-    const int s = (int)(c % slots);
+    const int sl = (int)(c % slots);
     const int64_t first = c * per_chunk;
     const int64_t cnt = (first + per_chunk <= num_arrays) ? per_chunk : num_arrays - first;
     float* h = h_data + first * array_len;
-    e = cudaMemcpyAsync(buf[s], h, cnt * row, cudaMemcpyHostToDevice, st[s]);
+    e = cudaMemcpyAsync(hs.buf[sl], h, cnt * row, cudaMemcpyHostToDevice, hs.st[sl]);
     if (e != cudaSuccess) break;
-    status = gas_sort_arrays(buf[s], cnt, array_len, st[s]);
+    status = gas_sort_arrays(hs.buf[sl], cnt, array_len, hs.st[sl]);
     if (status != GAS_SUCCESS) break;
-    e = cudaMemcpyAsync(h, buf[s], cnt * row, cudaMemcpyDeviceToHost, st[s]);
+    e = cudaMemcpyAsync(h, hs.buf[sl], cnt * row, cudaMemcpyDeviceToHost, hs.st[sl]);
   }
-  for (int s = 0; s < slots; ++s) {
-    if (st[s]) {
-      const cudaError_t e2 = cudaStreamSynchronize(st[s]);
-      if (e == cudaSuccess) e = e2;
-      cudaStreamDestroy(st[s]);
-    }
-    if (buf[s]) cudaFree(buf[s]);
+  for (int sl = 0; sl < slots; ++sl) {
+    const cudaError_t e2 = cudaStreamSynchronize(hs.st[sl]);
+    if (e == cudaSuccess) e = e2;
   }
   if (status != GAS_SUCCESS) return status;
   if (e != cudaSuccess) return cuda_fail(e);
