@@ -67,6 +67,42 @@ def _insertion_sort(seq: list) -> list:
     return seq
 
 
+def paper_method_phases(row_bits: np.ndarray) -> dict:
+    """The intermediate structures of Alg. 1-3 for ONE array (see paper_method_sort)."""
+    A = [int(v) for v in np.asarray(row_bits, dtype=np.uint32)]
+    n = len(A)
+    p = max(1, n // 20)
+    q = p - 1
+    samples = A[0::10]
+    m = len(samples)
+    sorted_samples = _insertion_sort(list(samples))
+    sp = [sorted_samples[((k + 1) * m) // p] for k in range(q)]
+    buckets = []
+    for t in range(p):
+        lo = sp[t - 1] if t > 0 else None
+        hi = sp[t] if t < q else None
+        buckets.append([x for x in A if (lo is None or _less(lo, x)) and (hi is None or not _less(hi, x))])
+    out = [x for b in buckets for x in _insertion_sort(list(b))]
+    return {"p": p, "q": q, "samples": samples, "sorted_samples": sorted_samples, "splitters": sp,
+            "z": [len(b) for b in buckets], "buckets": buckets, "output": out}
+
+
+def sta_steps(arrays):
+    """STA on a small list of arrays, returning every intermediate."""
+    tags = [i + 1 for i, a in enumerate(arrays) for _ in a]
+    vals = [x for a in arrays for x in a]
+    order = sorted(range(len(vals)), key=lambda j: tkey(vals[j]))          # stable sort by value
+    v1, t1 = [vals[j] for j in order], [tags[j] for j in order]
+    order2 = sorted(range(len(v1)), key=lambda j: t1[j])                   # stable sort by tag
+    v2, t2 = [v1[j] for j in order2], [t1[j] for j in order2]
+    out, pos = [], 0
+    for a in arrays:
+        out.append(v2[pos:pos + len(a)])
+        pos += len(a)
+    return {"tags_merged": tags, "values_merged": vals, "after_value_sort": (v1, t1),
+            "after_tag_sort": (v2, t2), "output": out}
+
+
 def paper_method_sort(row_bits: np.ndarray) -> np.ndarray:
     """GPU-ArraySort's three phases for ONE array, sequentially on the CPU.
 

@@ -336,3 +336,20 @@ def test_config2_ten_million_arrays_64bit_indexing():
     expect = oracle_sorted(datagen.rows("paper_uniform", seed, rows, n))
     got = x[torch.from_numpy(rows).to(DEV)].view(torch.int32).cpu().numpy().view(np.uint32)
     np.testing.assert_array_equal(got, expect)
+
+
+def test_tma_prefetch_variant_parity(monkeypatch):
+    """The opt-in TMA bulk-prefetch kernel (GAS_TMA=1) is part of the library: same parity bar."""
+    monkeypatch.setenv("GAS_TMA", "1")
+    for dist, N in (("special_mix", 3001), ("uniform_bits", 17)):
+        host = datagen.fixed(dist, 501, 0, N, 1000)
+        np.testing.assert_array_equal(gpu_sort_fixed(host, lead=4), oracle_sorted(host))
+
+
+def test_figure1_worked_example_on_gpu():
+    """The hand-worked Fig. 1 replica (tests/golden) through the C ABI."""
+    import json
+    import os
+    g = json.load(open(os.path.join(os.path.dirname(__file__), "golden", "fig1_gpu_arraysort_worked_example.json")))
+    host = np.array(g["input"], dtype=np.float32).view(np.uint32).reshape(1, -1)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), np.array(g["output"], dtype=np.float32).view(np.uint32)[None])

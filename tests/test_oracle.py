@@ -222,3 +222,47 @@ def test_pairs_stable():
         for kv in np.unique(k2[i]):
             sel = v2[i][k2[i] == kv]
             assert np.all(np.diff(sel.astype(np.int64)) > 0)
+
+
+# ------------------------------------------------ worked examples (figure replicas)
+
+
+def _f32_bits(xs):
+    return np.array(xs, dtype=np.float32).view(np.uint32)
+
+
+def test_fig1_worked_example():
+    """Hand-worked replica of Fig. 1 / Alg. 1-3 (tests/golden/fig1_*.json)."""
+    import json
+    g = json.load(open(os.path.join(os.path.dirname(__file__), "golden", "fig1_gpu_arraysort_worked_example.json")))
+    row = _f32_bits(g["input"])
+    ph = routes.paper_method_phases(row)
+    as_f = lambda xs: [float(np.uint32(x).view(np.float32)) for x in xs]  # noqa: E731
+    assert ph["p"] == g["p_buckets"] and ph["q"] == g["q_splitters"]
+    assert as_f(ph["samples"]) == g["samples"]
+    assert as_f(ph["sorted_samples"]) == g["sorted_samples"]
+    assert as_f(ph["splitters"]) == g["splitters"]
+    assert ph["z"] == g["z_bucket_sizes"]
+    assert [as_f(b) for b in ph["buckets"]] == g["buckets_after_phase2"]
+    assert as_f(ph["output"]) == g["output"]
+    a = row.reshape(1, -1).copy()
+    oracle.sort_arrays_(a)
+    np.testing.assert_array_equal(a[0], _f32_bits(g["output"]))
+
+
+def test_fig3_sta_worked_example():
+    """Hand-worked replica of Fig. 3 / the STA steps (tests/golden/fig3_*.json)."""
+    import json
+    g = json.load(open(os.path.join(os.path.dirname(__file__), "golden", "fig3_sta_worked_example.json")))
+    arrays = [[int(b) for b in _f32_bits(a)] for a in g["arrays"]]
+    st = routes.sta_steps(arrays)
+    as_f = lambda xs: [float(np.uint32(x).view(np.float32)) for x in xs]  # noqa: E731
+    assert st["tags_merged"] == g["tags_merged"]
+    assert as_f(st["values_merged"]) == g["values_merged"]
+    assert as_f(st["after_value_sort"][0]) == g["after_value_sort"]["values"]
+    assert st["after_value_sort"][1] == g["after_value_sort"]["tags"]
+    assert as_f(st["after_tag_sort"][0]) == g["after_tag_sort"]["values"]
+    assert st["after_tag_sort"][1] == g["after_tag_sort"]["tags"]
+    a = np.stack([_f32_bits(x) for x in g["arrays"]])
+    oracle.sort_arrays_(a)
+    np.testing.assert_array_equal(a, np.stack([_f32_bits(x) for x in g["output"]]))
