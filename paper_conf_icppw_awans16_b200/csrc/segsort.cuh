@@ -28,8 +28,11 @@ namespace gas {
 #define GAS_WARP_BLOCK 256
 #endif
 constexpr int kWarpBlock = GAS_WARP_BLOCK;  // threads per block for the warp-level classes
+#ifndef GAS_WARP_WARPS_PER_SM
+#define GAS_WARP_WARPS_PER_SM 16  // occupancy target of the warp classes: 16 warps/SM -> up to 128 registers
+#endif
 #ifndef GAS_WARP_MIN_BLOCKS
-#define GAS_WARP_MIN_BLOCKS (512 / GAS_WARP_BLOCK)  // 16 warps/SM -> up to 128 registers (no spills)
+#define GAS_WARP_MIN_BLOCKS (GAS_WARP_WARPS_PER_SM * 32 / GAS_WARP_BLOCK)
 #endif
 
 // XOR swizzle of 16-byte chunks inside 128-byte rows: chunk c of a rank-order
@@ -208,13 +211,17 @@ __global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS)
   }
 }
 
+#ifndef GAS_CTA_WARPS_PER_SM
+#define GAS_CTA_WARPS_PER_SM 20  // occupancy target (measured: 20 > 16, 24, 12) of the CTA classes (register budget 65536 / (32 x this))
+#endif
+
 template <int W, int WR>
 constexpr int cta_smem_bytes() { return 1024 * W * 4 + WR * 4096; }
 
 // CTA-level classes: P = 1024 * W (W = 2, 4, 8, 16), one array per CTA of 32*WR
 // threads (WR <= W real warps: n <= 1024 * WR, see sort_cta).
 template <int W, int WR, bool VEC>
-__global__ void __launch_bounds__(32 * WR, (16 / WR > 0 ? 16 / WR : 1)) k_fixed_cta(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+__global__ void __launch_bounds__(32 * WR, (GAS_CTA_WARPS_PER_SM / WR > 0 ? GAS_CTA_WARPS_PER_SM / WR : 1)) k_fixed_cta(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   constexpr int KPT = 32, T = 32 * WR, P = KPT * 32 * W;
   // dynamic shared memory (cta_smem_bytes<W, WR>()): P words of cross-warp
   // exchange / rank-order staging, then a 4 KB transpose scratch per warp
@@ -309,7 +316,7 @@ __global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS) k_offsets_war
 }
 
 template <int W, int WR>
-__global__ void __launch_bounds__(32 * WR, (16 / WR > 0 ? 16 / WR : 1)) k_offsets_cta(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
+__global__ void __launch_bounds__(32 * WR, (GAS_CTA_WARPS_PER_SM / WR > 0 ? GAS_CTA_WARPS_PER_SM / WR : 1)) k_offsets_cta(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
                                                          int64_t N, int64_t LO, int64_t HI,
                                                          unsigned long long* __restrict__ ctr, uint32_t one) {
   // handles the arrays with LO < length <= HI (HI <= 1024 * WR)
