@@ -35,6 +35,12 @@ constexpr int kWarpBlock = GAS_WARP_BLOCK;  // threads per block for the warp-le
 #define GAS_WARP_MIN_BLOCKS (GAS_WARP_WARPS_PER_SM * 32 / GAS_WARP_BLOCK)
 #endif
 
+// Occupancy target per class (blocks of kWarpBlock threads per SM), measured
+// on B200 (profiles/r01_variants_small_occupancy.txt): the 1024 class (G = 32)
+// and the 256 class (G = 8) run best at 2 blocks (<= 128 registers), the
+// others at 3 blocks (<= 85 registers, small spills).
+constexpr int warp_min_blocks(int G) { return (G == 32 || G == 8) ? GAS_WARP_MIN_BLOCKS : GAS_WARP_MIN_BLOCKS + 1; }
+
 // XOR swizzle of 16-byte chunks inside 128-byte rows: chunk c of a rank-order
 // buffer lives at physical chunk swz(c). Writes of 8 consecutive chunks per
 // thread and reads of 32 consecutive chunks per warp are both conflict-free.
@@ -107,7 +113,7 @@ __device__ __forceinline__ void stage_out_words(const uint32_t (&k)[KPT], uint4*
 
 // Warp-level classes: P = KPT * G <= 1024, GROUPS = 32 / G arrays per warp.
 template <int KPT, int G, bool VEC>
-__global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS) k_fixed_warp(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+__global__ void __launch_bounds__(kWarpBlock, warp_min_blocks(G)) k_fixed_warp(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   constexpr int GROUPS = 32 / G;
   constexpr int P = KPT * G;
   constexpr int WORDS = 32 * KPT;  // per warp
@@ -268,7 +274,7 @@ __device__ __forceinline__ bool in_class(int64_t len, int P) {
 }
 
 template <int KPT, int G>
-__global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS) k_offsets_warp(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
+__global__ void __launch_bounds__(kWarpBlock, warp_min_blocks(G)) k_offsets_warp(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
                                                           int64_t N, uint32_t one) {
   constexpr int GROUPS = 32 / G;
   constexpr int P = KPT * G;
