@@ -35,6 +35,10 @@ constexpr int kWarpBlock = GAS_WARP_BLOCK;  // threads per block for the warp-le
 #define GAS_WARP_MIN_BLOCKS (GAS_WARP_WARPS_PER_SM * 32 / GAS_WARP_BLOCK)
 #endif
 
+#ifndef GAS_SMALL_PREFETCH
+#define GAS_SMALL_PREFETCH 1
+#endif
+
 // Occupancy target per class (blocks of kWarpBlock threads per SM), measured
 // on B200 (profiles/r01_variants_small_occupancy.txt): the 1024 class (G = 32)
 // and the 256 class (G = 8) run best at 2 blocks (<= 128 registers), the
@@ -127,6 +131,20 @@ __global__ void __launch_bounds__(kWarpBlock, warp_min_blocks(G)) k_fixed_warp(u
     const bool valid = a < N;
     uint32_t k[KPT];
     load_keys<KPT, G, VEC>(k, d + (valid ? a : 0) * (int64_t)n, n, g, valid);
+#if GAS_SMALL_PREFETCH
+    if constexpr (VEC && G >= 8 && G < 32) {
+      // P = 256, 512: several arrays per warp, little work per byte, exposed to
+      // HBM latency: warm L2 with the warp's next GROUPS arrays (one contiguous
+      // TMA bulk prefetch issued by one lane). Measured: n=500 6.85 -> 6.35 ms;
+      // no gain for the other classes (profiles/r01_variants_small_prefetch.txt).
+      const int64_t nb = base + nwarps * GROUPS;
+      if (lane == 0 && nb < N) {
+        const int64_t cnt = (N - nb < GROUPS) ? N - nb : GROUPS;
+        asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + nb * (int64_t)n),
+                     "r"((uint32_t)(cnt * n * 4)) : "memory");
+      }
+    }
+#endif
     if constexpr (KPT == 32 && G >= 2) sort_group_warp<G>(k, g, reinterpret_cast<uint32_t*>(sb), one);
     else Bitonic<KPT, G, 1>::sort(k, g, 0, nullptr, one);
     stage_out_words<KPT>(k, sb, grp * P + g * KPT);
