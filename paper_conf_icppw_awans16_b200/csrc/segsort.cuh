@@ -132,16 +132,19 @@ __global__ void __launch_bounds__(kWarpBlock, warp_min_blocks(G)) k_fixed_warp(u
     uint32_t k[KPT];
     load_keys<KPT, G, VEC>(k, d + (valid ? a : 0) * (int64_t)n, n, g, valid);
 #if GAS_SMALL_PREFETCH
-    if constexpr (VEC && G >= 8 && G < 32) {
+    if constexpr (G >= 8 && G < 32) {
       // P = 256, 512: several arrays per warp, little work per byte, exposed to
       // HBM latency: warm L2 with the warp's next GROUPS arrays (one contiguous
       // TMA bulk prefetch issued by one lane). Measured: n=500 6.85 -> 6.35 ms;
       // no gain for the other classes (profiles/r01_variants_small_prefetch.txt).
+      // (unaligned rows: only the 16-byte-aligned interior of the range)
       const int64_t nb = base + nwarps * GROUPS;
       if (lane == 0 && nb < N) {
         const int64_t cnt = (N - nb < GROUPS) ? N - nb : GROUPS;
-        asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + nb * (int64_t)n),
-                     "r"((uint32_t)(cnt * n * 4)) : "memory");
+        const uintptr_t lo = (reinterpret_cast<uintptr_t>(d + nb * (int64_t)n) + 15) & ~uintptr_t(15);
+        const uintptr_t hi = reinterpret_cast<uintptr_t>(d + (nb + cnt) * (int64_t)n) & ~uintptr_t(15);
+        if (hi > lo)
+          asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(lo), "r"((uint32_t)(hi - lo)) : "memory");
       }
     }
 #endif
