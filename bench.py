@@ -333,10 +333,11 @@ def main():
     torch.cuda.synchronize()
 
     evs = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
-    barrier()
-    torch.cuda.synchronize()
-    launches0 = gas.launch_count()
     with ClockSampler(local) as clk:
+        time.sleep(0.05)  # let the NVML sampler thread start before the timed region (it shares the GIL)
+        barrier()
+        torch.cuda.synchronize()
+        launches0 = gas.launch_count()
         t_wall0 = time.perf_counter()
         for s in range(args.steps):
             work.copy_(pristine)  # untimed restore: the sort is in place

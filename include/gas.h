@@ -20,7 +20,7 @@
  * Conventions for every entry point:
  *   - Pointers named d_* are DEVICE memory of the current device, owned by
  *     the caller; gas_sort_arrays and gas_sort_pairs allocate nothing (zero
- *     workspace); the offsets variant uses 56 bytes (see there); the library
+ *     workspace); the offsets variant keeps 56 bytes per stream (see there); the library
  *     never calls cudaSetDevice.
  *   - Work is enqueued on `stream` (0 = legacy default stream) and the call
  *     returns without a host synchronisation. Argument and launch-
@@ -77,8 +77,9 @@ gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len,
  *                  on the device first (with a stream synchronisation) and a
  *                  violation returns GAS_ERROR_INVALID_VALUE with nothing sorted.
  *   max_array_len > gas_max_array_len(): GAS_ERROR_UNSUPPORTED.
- * Workspace: 56 bytes of stream-ordered device memory (cudaMallocAsync /
- * cudaFreeAsync on `stream`) for dynamic scheduling when max_array_len > 1024.
+ * Workspace: 56 bytes of device memory per (device, stream) for dynamic
+ * scheduling when max_array_len > 1024, allocated on the first such call and
+ * kept (re-zeroed in stream order by every call).
  * One kernel launch per size class up to max_array_len (at most 17 launches:
  * powers of two up to 2048, then (2048,3072], (3072,4096], (4096,6144],
  * (6144,8192], (8192,12288], (12288,16384]).

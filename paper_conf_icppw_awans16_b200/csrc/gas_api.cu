@@ -1,6 +1,7 @@
 // gas_api.cu — the C ABI of include/gas.h: argument validation, size-class
 // dispatch, launch configuration and status codes.
 #include <atomic>
+#include <map>
 #include <mutex>
 #include <cstdint>
 #include <cstdlib>
@@ -247,6 +248,25 @@ struct HostStaging {
 };
 HostStaging g_staging[kMaxDevices];
 
+// Per-(device, stream) window counters of the offsets variant (see there).
+constexpr int kCounters = 7;
+std::mutex g_ctr_mu;
+std::map<std::pair<int, cudaStream_t>, unsigned long long*> g_ctr;
+
+cudaError_t counters_for(cudaStream_t stream, unsigned long long** out) {
+  int dev = 0;
+  cudaError_t e = cudaGetDevice(&dev);
+  if (e != cudaSuccess) return e;
+  std::lock_guard<std::mutex> lock(g_ctr_mu);
+  auto& slot = g_ctr[{dev, stream}];
+  if (!slot) {
+    e = cudaMalloc(&slot, kCounters * sizeof(unsigned long long));
+    if (e != cudaSuccess) { slot = nullptr; return e; }
+  }
+  *out = slot;
+  return cudaSuccess;
+}
+
 bool env_check() {
   const char* v = std::getenv("GAS_CHECK");
   return v && std::strcmp(v, "0") != 0 && v[0] != '\0';
@@ -293,11 +313,13 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
     if (h) return GAS_ERROR_INVALID_VALUE;
   }
   uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
-  // 7 window counters for the CTA classes' dynamic scheduling (stream-ordered, 56 bytes)
+  // 7 window counters for the CTA classes' dynamic scheduling: 56 bytes per
+  // (device, stream), allocated on first use and re-zeroed in stream order by
+  // every call (calls on one stream are ordered; different streams never share)
   unsigned long long* ctr = nullptr;
   if (max_array_len > 1024) {
-    cudaError_t e = cudaMallocAsync(&ctr, 7 * sizeof(unsigned long long), stream);
-    if (e == cudaSuccess) e = cudaMemsetAsync(ctr, 0, 7 * sizeof(unsigned long long), stream);
+    cudaError_t e = counters_for(stream, &ctr);
+    if (e == cudaSuccess) e = cudaMemsetAsync(ctr, 0, kCounters * sizeof(unsigned long long), stream);
     if (e != cudaSuccess) return cuda_fail(e);
   }
   // size classes: 2, 4, ..., 2048 (len in (P/2, P]), then (2048, 3072] and (3072, 4096]
@@ -306,15 +328,8 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
   for (int c = 0; c < 17; ++c) {
     if (lower[c] >= max_array_len) break;
     const cudaError_t e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, ctr, stream);
-    if (e != cudaSuccess) {
-      if (ctr) cudaFreeAsync(ctr, stream);
-      return cuda_fail(e);
-    }
-    g_launches.fetch_add(1, std::memory_order_relaxed);
-  }
-  if (ctr) {
-    const cudaError_t e = cudaFreeAsync(ctr, stream);
     if (e != cudaSuccess) return cuda_fail(e);
+    g_launches.fetch_add(1, std::memory_order_relaxed);
   }
   return GAS_SUCCESS;
 }
