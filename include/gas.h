@@ -31,6 +31,10 @@
  *     2^31 elements (e.g. 10^7 x 1000).
  *   - Functions are reentrant and thread-safe; concurrent calls on
  *     overlapping memory are the caller's race.
+ *   - The device-resident entry points enqueue only kernels (and, for the
+ *     offsets variant, one memset) on `stream`: after one warm-up call on a
+ *     stream they can be captured into a CUDA graph and replayed
+ *     (tests/test_gpu_parity.py::test_cuda_graph_capture_and_replay).
  *   - No C++ exceptions cross this boundary.
  */
 #ifndef GAS_H

@@ -353,3 +353,33 @@ def test_figure1_worked_example_on_gpu():
     g = json.load(open(os.path.join(os.path.dirname(__file__), "golden", "fig1_gpu_arraysort_worked_example.json")))
     host = np.array(g["input"], dtype=np.float32).view(np.uint32).reshape(1, -1)
     np.testing.assert_array_equal(gpu_sort_fixed(host), np.array(g["output"], dtype=np.float32).view(np.uint32)[None])
+
+
+def test_cuda_graph_capture_and_replay():
+    """The device-resident entry points enqueue only kernels/memsets on the given
+    stream (no host sync, no allocation once warm), so they can be captured in a
+    CUDA graph and replayed (serving-style use)."""
+    N, n = 5000, 1000
+    host = datagen.fixed("special_mix", 601, 0, N, n)
+    x = torch.from_numpy(host.copy().view(np.float32)).to(DEV)
+    lens = datagen.lengths(602, 0, 2000, 100, 4000)
+    off = datagen.offsets_from_lengths(lens)
+    rdata = datagen.ragged("spectra_mz", 602, 0, off)
+    r = torch.from_numpy(rdata.view(np.int32).copy()).to(DEV)
+    off_d = torch.from_numpy(off).to(DEV)
+    s = torch.cuda.Stream()
+    with torch.cuda.stream(s):  # warm-up outside capture (per-stream counters are allocated here)
+        gas.gas_sort_arrays(x.clone())
+        gas.gas_sort_arrays_offsets(r.clone().view(torch.float32), off_d, 4000)
+    s.synchronize()
+    g = torch.cuda.CUDAGraph()
+    with torch.cuda.graph(g, stream=s):
+        gas.gas_sort_arrays(x)
+        gas.gas_sort_arrays_offsets(r.view(torch.float32), off_d, 4000)
+    for _ in range(2):  # replays: first sorts, second re-sorts sorted data (idempotent)
+        g.replay()
+    torch.cuda.synchronize()
+    np.testing.assert_array_equal(to_host(x.view(torch.int32)).reshape(N, n), oracle_sorted(host))
+    expect = rdata.copy()
+    oracle.sort_arrays_offsets_(expect, off)
+    np.testing.assert_array_equal(to_host(r), expect)
