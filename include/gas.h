@@ -109,7 +109,8 @@ gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays,
  * chunks (host->device copy, sort, device->host copy on rotating streams so
  * the two copy directions and the sort overlap) and the sorted batch is
  * written back to h_data. Pinned (page-locked) host memory gives full-duplex
- * PCIe; pageable memory works but is slower. BLOCKING: returns after the
+ * PCIe; pageable memory works but is much slower (measured for 2M x 1000 on
+ * one B200: 175 ms pinned, 1.14 s pageable — register or pin the buffer). BLOCKING: returns after the
  * result is in h_data. Device staging (3 x 128 MB by default, GAS_HOST_CHUNK_MB /
  * GAS_HOST_SLOTS) and its streams are allocated on first use per device and kept
  * for later calls; concurrent host-path calls on one device are serialised.
