@@ -1,0 +1,324 @@
+// bucket1024.cuh — bucket-then-network sort of one array of 512 < n <= 1024
+// keys by one warp (the n = 1000 headline of BASELINE.json configs[1]).
+//
+// Why: the pure sorting network of warp1024.cuh spends ~26 compare-exchanges
+// per key (levels 6-10 of a 1024-key merge network) and is bound by the
+// integer-ALU pipe and instruction issue. This kernel first
+// splits the array into 62 value ranges — the paper's own idea of
+// data-independent buckets whose concatenation is the sorted array with no
+// merge step (§4.1, Alg. 2 P:L250-297 §5.2) — and then sorts each
+// bucket (<= 32 keys) with the 191-comparator odd-even network in one lane's
+// registers (6 compare-exchanges per key per bucket). Differences from the
+// paper, for B200: buckets come from linear interpolation between the array's
+// min and max (one FADD + one FFMA per key on the FMA pipe) instead of a
+// sorted sample and per-thread splitter scans (Alg. 1-2); ranks come from
+// conflict-free per-lane shared-memory counters and one rotated prefix scan
+// instead of a global bucket-size array Z (Def. 4); nothing but
+// the array itself touches HBM.
+//
+// Correctness does not depend on the data: the bucket map
+//     b(v) = rn(rn(v - vmin) * s + 2^23) - 2^23,   s = rn(61 / rn(vmax - vmin))
+// is monotone non-decreasing in v (every step is a monotone rounding of a
+// monotone function), so every key of bucket b precedes (in IEEE totalOrder,
+// DESIGN.md reading C-1) every key of bucket b+1, and ±0 (equal values) share
+// a bucket whose network orders them. 0 <= b <= 61 because rn(v - vmin) lies
+// in [0, rn(vmax - vmin)] and range * s <= 61 (1 + 2^-24) < 61.5.
+// The warp falls back to the full network (warp1024.cuh) for the whole array
+// when the map cannot be used — a NaN or an infinity in the array, all values
+// equal, a range that overflows or underflows — or when a bucket would hold
+// more than 32 keys (measured on the paper's uniform data: 0.5% of arrays).
+// The decision is warp-uniform, so both paths are branch-free inside a warp.
+#pragma once
+#include <cstdint>
+
+#include "bitonic.cuh"
+#include "ordered_key.cuh"
+#include "warp1024.cuh"
+
+namespace gas {
+
+constexpr int kBkBuckets = 62;  // value-interpolation buckets 0..61 (rows 62, 63 stay empty)
+#ifndef GAS_BK_BLOCK
+#define GAS_BK_BLOCK 128
+#endif
+#ifndef GAS_BK_WARPS_PER_SM
+#define GAS_BK_WARPS_PER_SM 16
+#endif
+#ifndef GAS_BK_PAIRCOUNT
+#define GAS_BK_PAIRCOUNT 1
+#endif
+#ifndef GAS_BK_PREFETCH
+#define GAS_BK_PREFETCH 1
+#endif
+constexpr int kBkBlock = GAS_BK_BLOCK;
+// Per warp: u16 counters [64 rows (bucket)][32 lanes] (4 KB) — reused as the
+// position-order output staging buffer (n <= 1024 words) — then the slot
+// buffer [32 positions][64 buckets] of u32 keys (8 KB), also the 4 KB
+// transpose scratch of the fallback network.
+constexpr int kBkCntBytes = 64 * 32 * 2;
+constexpr int kBkSlotBytes = 32 * 64 * 4;
+constexpr int kBkWarpBytes = kBkCntBytes + kBkSlotBytes;
+constexpr int kBkSmemBytes = (kBkBlock / 32) * kBkWarpBytes;
+
+__device__ __forceinline__ float fmin_nan(float a, float b) {
+  float r;
+  asm("min.NaN.f32 %0, %1, %2;" : "=f"(r) : "f"(a), "f"(b));
+  return r;
+}
+__device__ __forceinline__ float fmax_nan(float a, float b) {
+  float r;
+  asm("max.NaN.f32 %0, %1, %2;" : "=f"(r) : "f"(a), "f"(b));
+  return r;
+}
+__device__ __forceinline__ uint32_t lds16(uint32_t a) {
+  uint16_t v;
+  asm volatile("ld.shared.u16 %0, [%1];" : "=h"(v) : "r"(a) : "memory");
+  return v;
+}
+__device__ __forceinline__ void sts16(uint32_t a, uint32_t v) {
+  asm volatile("st.shared.u16 [%0], %1;" ::"r"(a), "h"((uint16_t)v) : "memory");
+}
+__device__ __forceinline__ uint32_t lds32(uint32_t a) {
+  uint32_t v;
+  asm volatile("ld.shared.u32 %0, [%1];" : "=r"(v) : "r"(a) : "memory");
+  return v;
+}
+__device__ __forceinline__ void sts32(uint32_t a, uint32_t v) {
+  asm volatile("st.shared.u32 [%0], %1;" ::"r"(a), "r"(v) : "memory");
+}
+__device__ __forceinline__ uint4 lds128(uint32_t a) {
+  uint4 v;
+  asm volatile("ld.shared.v4.u32 {%0, %1, %2, %3}, [%4];" : "=r"(v.x), "=r"(v.y), "=r"(v.z), "=r"(v.w) : "r"(a) : "memory");
+  return v;
+}
+__device__ __forceinline__ void sts128(uint32_t a, uint4 v) {
+  asm volatile("st.shared.v4.u32 [%0], {%1, %2, %3, %4};" ::"r"(a), "r"(v.x), "r"(v.y), "r"(v.z), "r"(v.w) : "memory");
+}
+
+// Bucket map of one value (see the header comment): the bits of
+// rn(rn(v - vmin) * s + 2^23) are 0x4B000000 + b.
+__device__ __forceinline__ uint32_t bucket_bits(uint32_t raw, float vmin, float s) {
+  const float dv = __fsub_rn(__uint_as_float(raw), vmin);
+  return __float_as_uint(__fmaf_rn(dv, s, 8388608.0f));
+}
+
+// The whole-array network (warp1024.cuh) for arrays the bucket map cannot
+// handle; out of line so that the bucket path's hot code stays compact.
+__device__ __noinline__ void bucket1024_fallback(uint32_t (&k)[32], uint4* dst, int nc, int lane, uint32_t* scratch,
+                                                 uint32_t one) {
+  __syncwarp();
+#pragma unroll
+  for (int q = 0; q < 8; ++q) {
+    const bool valid = q < 4 || lane + 32 * q < nc;
+#pragma unroll
+    for (int j = 0; j < 4; ++j) k[4 * q + j] = valid ? key_from_bits(k[4 * q + j]) : kPadKey;
+  }
+  sort1024_warp(k, lane, scratch, one);
+  uint4* sb = reinterpret_cast<uint4*>(scratch);
+  stage_out<32>(k, sb, lane * 8);
+  __syncwarp();
+#pragma unroll
+  for (int q = 0; q < 8; ++q) {
+    const int c = lane + 32 * q;
+    if (c < nc) st_stream(dst + c, sb[swz(c)]);
+  }
+}
+
+// Fixed-length arrays, 512 < n <= 1024, 16-byte-aligned rows (n % 4 == 0).
+// One warp per array (persistent grid-stride).
+__global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
+    k_fixed_bucket1024(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+  extern __shared__ __align__(16) uint4 bk_smem[];
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
+  const uint32_t cnt_sa = wsa;                 // u16 counter (b, lane) at cnt_sa + b*64 + lane*2
+  const uint32_t slot_sa = wsa + kBkCntBytes;  // slot (p, b) at slot_sa + (p*64 + b)*4
+  uint32_t* const slot_ptr = reinterpret_cast<uint32_t*>(reinterpret_cast<unsigned char*>(bk_smem) +
+                                                         warp * kBkWarpBytes + kBkCntBytes);
+  const int nc = n >> 2;  // 16-byte chunks per array (> 128)
+  const int64_t nwarps = (int64_t)gridDim.x * (kBkBlock / 32);
+  // counting address of bucket bits tb for this lane: cnt_sa + b*64 + lane*2
+  const uint32_t cnt_lane0 = cnt_sa + lane * 2 - 0x4B000000u * 64u;
+  const uint32_t slot_b0 = slot_sa - 0x4B000000u * 4u;
+
+  for (int64_t a = (int64_t)blockIdx.x * (kBkBlock / 32) + warp; a < N; a += nwarps) {
+    uint4* const dst = reinterpret_cast<uint4*>(d + a * (int64_t)n);
+    // ---- a2: stage in (raw bits). Pad slots repeat a real value of the lane
+    // (neutral for min/max) and are excluded from counting and scatter.
+    uint32_t k[32];
+    {
+      const uint4 v0 = ld_stream(dst + lane);
+      k[0] = v0.x; k[1] = v0.y; k[2] = v0.z; k[3] = v0.w;
+#pragma unroll
+      for (int q = 1; q < 8; ++q) {
+        const int c = lane + 32 * q;
+        uint4 v = make_uint4(v0.x, v0.x, v0.x, v0.x);
+        if (q < 4 || c < nc) v = ld_stream(dst + c);
+        k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
+      }
+    }
+#if GAS_BK_PREFETCH
+    if (lane == 0 && a + nwarps < N)  // warm L2 with this warp's next array (one TMA bulk prefetch)
+      asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + (a + nwarps) * (int64_t)n),
+                   "r"((uint32_t)n * 4u) : "memory");
+#endif
+    // ---- bucket map parameters: min and max value (NaN-propagating)
+    float vmin = __uint_as_float(k[0]), vmax = vmin;
+#pragma unroll
+    for (int r = 1; r < 32; ++r) {
+      vmin = fmin_nan(vmin, __uint_as_float(k[r]));
+      vmax = fmax_nan(vmax, __uint_as_float(k[r]));
+    }
+#pragma unroll
+    for (int m = 16; m >= 1; m >>= 1) {
+      vmin = fmin_nan(vmin, __shfl_xor_sync(0xffffffffu, vmin, m));
+      vmax = fmax_nan(vmax, __shfl_xor_sync(0xffffffffu, vmax, m));
+    }
+    const float range = __fsub_rn(vmax, vmin);
+    const float s = __fdiv_rn(61.0f, range);
+    // finite min and max (no NaN, no inf), distinct, finite range and scale
+    bool use_buckets = fabsf(vmin) <= 3.402823466e38f && fabsf(vmax) <= 3.402823466e38f && range > 0.0f &&
+                       range <= 3.402823466e38f && s <= 3.402823466e38f;
+    uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
+    uint32_t rk[32];
+    if (use_buckets) {
+      // slot buffer <- pad keys, counters <- 0 (the previous array is done with both)
+#pragma unroll
+      for (int q = 0; q < kBkSlotBytes / 16 / 32; ++q)
+        sts128(slot_sa + (lane + 32 * q) * 16, make_uint4(kPadKey, kPadKey, kPadKey, kPadKey));
+#pragma unroll
+      for (int q = 0; q < kBkCntBytes / 16 / 32; ++q) sts128(cnt_sa + (lane + 32 * q) * 16, make_uint4(0, 0, 0, 0));
+      __syncwarp();
+      // ---- count: per-lane u16 counters, column `lane` of row b (conflict-free).
+      // Keys go in pairs so that the load -> increment -> store chain through
+      // shared memory has 16 links instead of 32: both counters are loaded
+      // first, and if both keys hit the same counter the second count is the
+      // first + 1 (the later store then leaves the right total).
+#pragma unroll
+      for (int r = 0; r < 32; r += 2) {
+        const int q = r >> 2;
+        if (q < 4 || lane + 32 * q < nc) {
+          const uint32_t ca = bucket_bits(k[r], vmin, s) * 64u + cnt_lane0;
+#if GAS_BK_PAIRCOUNT
+          const uint32_t cb = bucket_bits(k[r + 1], vmin, s) * 64u + cnt_lane0;
+          const uint32_t c0 = lds16(ca);
+          uint32_t c1 = lds16(cb);
+          c1 = (ca == cb) ? c0 + 1 : c1;
+          sts16(ca, c0 + 1);
+          sts16(cb, c1 + 1);
+          rk[r] = c0;
+          rk[r + 1] = c1;
+#else
+          const uint32_t c0 = lds16(ca);
+          sts16(ca, c0 + 1);
+          rk[r] = c0;
+          const uint32_t cb = bucket_bits(k[r + 1], vmin, s) * 64u + cnt_lane0;
+          const uint32_t c1 = lds16(cb);
+          sts16(cb, c1 + 1);
+          rk[r + 1] = c1;
+#endif
+        } else {
+          rk[r] = 0;
+          rk[r + 1] = 0;
+        }
+      }
+      __syncwarp();
+      // ---- scan: lane l turns rows l and l+32 into exclusive offsets. The
+      // order of lanes inside a row is any fixed order (the chunks are read
+      // rotated by lane/2 to avoid bank conflicts; lo halves before hi halves).
+      uint4 w[2][4];
+#pragma unroll
+      for (int h = 0; h < 2; ++h)
+#pragma unroll
+        for (int q = 0; q < 4; ++q) w[h][q] = lds128(cnt_sa + (lane + 32 * h) * 64 + (((q + (lane >> 1)) & 3) << 4));
+      uint32_t tot[2];
+#pragma unroll
+      for (int h = 0; h < 2; ++h) {
+        uint32_t sum = 0;
+#pragma unroll
+        for (int q = 0; q < 4; ++q) sum += w[h][q].x + w[h][q].y + w[h][q].z + w[h][q].w;
+        const uint32_t tlo = sum & 0xFFFFu;
+        tot[h] = tlo + (sum >> 16);
+        uint32_t p = tlo << 16;
+#pragma unroll
+        for (int q = 0; q < 4; ++q) {
+          uint4 o;
+          o.x = p; p += w[h][q].x;
+          o.y = p; p += w[h][q].y;
+          o.z = p; p += w[h][q].z;
+          o.w = p; p += w[h][q].w;
+          w[h][q] = o;
+        }
+      }
+#pragma unroll
+      for (int h = 0; h < 2; ++h)
+#pragma unroll
+        for (int q = 0; q < 4; ++q) sts128(cnt_sa + (lane + 32 * h) * 64 + (((q + (lane >> 1)) & 3) << 4), w[h][q]);
+      t0 = tot[0];
+      t1 = tot[1];
+      use_buckets = __all_sync(0xffffffffu, t0 <= 32u && t1 <= 32u);
+      if (use_buckets) {
+        // bucket bases: exclusive scan of the 64 bucket sizes (two 16-bit halves)
+        uint32_t x = t0 | (t1 << 16);
+#pragma unroll
+        for (int m = 1; m < 32; m <<= 1) {
+          const uint32_t y = __shfl_up_sync(0xffffffffu, x, m);
+          if (lane >= m) x += y;
+        }
+        const uint32_t total_lo = __shfl_sync(0xffffffffu, x & 0xFFFFu, 31);
+        base0 = (x & 0xFFFFu) - t0;
+        base1 = total_lo + (x >> 16) - t1;
+        __syncwarp();
+        // ---- scatter: key of rank p in bucket b -> slot (p, b)
+#pragma unroll
+        for (int r = 0; r < 32; ++r) {
+          const int q = r >> 2;
+          if (q < 4 || lane + 32 * q < nc) rk[r] += lds16(bucket_bits(k[r], vmin, s) * 64u + cnt_lane0);
+        }
+#pragma unroll
+        for (int r = 0; r < 32; ++r) {
+          const int q = r >> 2;
+          if (q < 4 || lane + 32 * q < nc) {
+            const uint32_t sa = rk[r] * 256u + bucket_bits(k[r], vmin, s) * 4u + slot_b0;
+            sts32(sa, key_from_bits(k[r]));
+          }
+        }
+        __syncwarp();
+      }
+    }
+
+    if (use_buckets) {
+      // ---- per round rho = 0, 1: gather bucket b = lane + 32 rho (its column
+      // of the slot buffer, conflict-free), sort it in registers, and stage its
+      // keys at output words base_b + i, i < size_b, in the dead counter region
+      // (4 KB = 1024 words >= n). Each staging store is predicated: stores of
+      // one lane to distinct addresses may be reordered, so no write may rely
+      // on another lane's later write. The round loop is rolled to keep the hot
+      // code inside the instruction cache.
+      const uint32_t out_sa = cnt_sa;
+#pragma unroll 1
+      for (int rho = 0; rho < 2; ++rho) {
+        const uint32_t col = slot_sa + lane * 4 + rho * 128;
+        const uint32_t tb = rho ? t1 : t0;
+        const uint32_t ob = out_sa + (rho ? base1 : base0) * 4;
+#pragma unroll
+        for (int i = 0; i < 32; ++i) k[i] = lds32(col + i * 256);
+        sort32_regs(k, one);
+#pragma unroll
+        for (int i = 0; i < 32; ++i)
+          if ((uint32_t)i < tb) sts32(ob + i * 4, bits_from_key(k[i]));
+      }
+      __syncwarp();
+#pragma unroll
+      for (int q = 0; q < 8; ++q) {
+        const int c = lane + 32 * q;
+        if (c < nc) st_stream(dst + c, lds128(out_sa + c * 16));
+      }
+    } else {
+      bucket1024_fallback(k, dst, nc, lane, slot_ptr, one);
+    }
+    __syncwarp();
+  }
+}
+
+}  // namespace gas

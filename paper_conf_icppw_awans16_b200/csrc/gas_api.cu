@@ -11,6 +11,7 @@
 
 #include "../../include/gas.h"
 #include "segsort.cuh"
+#include "bucket1024.cuh"
 #include "pairs.cuh"
 
 namespace {
@@ -112,6 +113,23 @@ cudaError_t launch_fixed_1024_tma(uint32_t* d, int64_t N, int n, cudaStream_t s)
   return cudaGetLastError();
 }
 
+// Bucket-then-network kernel for 512 < n <= 1024 with aligned rows
+// (bucket1024.cuh). Default on; GAS_BUCKET=0 selects the pure network.
+cudaError_t launch_fixed_bucket1024(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  const cudaError_t attr = cudaFuncSetAttribute(gas::k_fixed_bucket1024, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                                gas::kBkSmemBytes);
+  if (attr != cudaSuccess) return attr;
+  const int grid = persistent_grid_smem(gas::k_fixed_bucket1024, gas::kBkBlock, gas::kBkSmemBytes,
+                                        (N + gas::kBkBlock / 32 - 1) / (gas::kBkBlock / 32));
+  gas::k_fixed_bucket1024<<<grid, gas::kBkBlock, gas::kBkSmemBytes, s>>>(d, N, n, 1u);
+  return cudaGetLastError();
+}
+
+bool bucket_enabled() {
+  const char* v = std::getenv("GAS_BUCKET");
+  return !(v && std::strcmp(v, "0") == 0);
+}
+
 template <bool VEC>
 cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   switch (size_class(n)) {
@@ -129,6 +147,7 @@ cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
       // global-load stalls but is 5% slower overall (profiles/r01_ab_tma.txt):
       // the kernel is ALU/issue-bound, not latency-bound.
       if (VEC && env_flag("GAS_TMA")) return launch_fixed_1024_tma(d, N, n, s);
+      if (VEC && bucket_enabled()) return launch_fixed_bucket1024(d, N, n, s);
       return launch_fixed_warp<32, 32, VEC>(d, N, n, s);
     default: return dispatch_fixed_cta<VEC>(d, N, n, s);
   }

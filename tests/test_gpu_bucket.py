@@ -1,0 +1,134 @@
+"""GPU parity of the bucket-then-network kernel (csrc/bucket1024.cuh), the
+default path for 512 < n <= 1024 with 16-byte-aligned rows, against the CPU
+oracle, bit-exact. Covers both of its warp-uniform branches: the bucket path
+(finite values, every bucket <= 32 keys) and the full-network fallback (NaN,
+inf, all-equal, overflowing or underflowing range, a bucket of 33 keys), and
+the edges of the bucket map (ties at bucket boundaries, ±0, subnormals).
+
+With vmin = 0 and vmax = 61 the map is b(v) = rint(v) (s = 61 / 61 = 1), which
+lets the tests put an exact number of keys into a chosen bucket."""
+import numpy as np
+import pytest
+
+import datagen
+import oracle
+
+torch = pytest.importorskip("torch")
+pytestmark = pytest.mark.gpu
+
+if not torch.cuda.is_available():  # pragma: no cover
+    pytest.skip("needs a GPU", allow_module_level=True)
+
+import paper_conf_icppw_awans16_b200 as gas  # noqa: E402
+
+from tests.test_gpu_parity import gpu_sort_fixed, oracle_sorted  # noqa: E402
+
+
+def f32(a) -> np.ndarray:
+    return np.asarray(a, dtype=np.float32).view(np.uint32)
+
+
+def spread_array(n: int, rng, heavy_bucket=None, heavy_count=0, heavy_values=None) -> np.ndarray:
+    """n values in [0, 61] with 0 and 61 present; optionally `heavy_count` keys
+    in bucket `heavy_bucket` (b = rint(v)); the rest spread over the other buckets."""
+    vals = [0.0, 61.0]
+    if heavy_bucket is not None:
+        hv = heavy_values if heavy_values is not None else np.full(heavy_count, float(heavy_bucket))
+        vals += list(hv)
+    rest = n - len(vals)
+    others = [b for b in range(1, 61) if b != heavy_bucket]
+    per = np.bincount(np.arange(rest) % len(others), minlength=len(others))
+    assert per.max() <= 24
+    for b, c in zip(others, per):
+        vals += list(b + rng.uniform(-0.45, 0.45, size=c))
+    v = np.array(vals, dtype=np.float32)
+    rng.shuffle(v)
+    return v.view(np.uint32)
+
+
+@pytest.mark.parametrize("n", [513, 516, 520, 772, 999, 1000, 1020, 1024])
+@pytest.mark.parametrize("dist", ["paper_uniform", "spectra_mz", "sorted", "reverse", "spectra_intensity",
+                                  "dup16", "special_mix", "uniform_bits"])
+def test_bucket_kernel_distributions(dist, n):
+    host = datagen.fixed(dist, 7001, 0, 700, n)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("count", [31, 32, 33, 40])
+def test_bucket_capacity_edge(count):
+    """A bucket with exactly 32 keys takes the bucket path, 33 the fallback: both exact."""
+    rng = np.random.default_rng(count)
+    rows = []
+    for i in range(64):
+        hv = 10.0 + rng.uniform(-0.49, 0.49, size=count).astype(np.float32)
+        rows.append(spread_array(1000, rng, heavy_bucket=10, heavy_count=count, heavy_values=hv))
+    host = np.stack(rows)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+def test_bucket_boundary_ties_and_signed_zeros():
+    """Values at x.5 (round-half-even boundaries of the map), duplicates and ±0."""
+    rng = np.random.default_rng(5)
+    rows = []
+    for i in range(50):
+        v = np.concatenate([[0.0, 61.0], np.arange(61) + 0.5, np.full(10, -0.0), np.full(10, 0.0),
+                            rng.integers(0, 62, size=1000 - 2 - 61 - 20).astype(np.float64)])
+        v = v.astype(np.float32)
+        rng.shuffle(v)
+        rows.append(v.view(np.uint32))
+    host = np.stack(rows)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+    # negative range with -0/+0 at the top
+    neg = -host.view(np.float32)
+    h2 = np.ascontiguousarray(neg).view(np.uint32)
+    np.testing.assert_array_equal(gpu_sort_fixed(h2), oracle_sorted(h2))
+
+
+def test_bucket_map_fallback_triggers():
+    """NaN, +-inf, all equal, range overflow (-3e38 .. 3e38), subnormal range
+    (scale overflows), a single distinct value among ±0: all take the fallback."""
+    rng = np.random.default_rng(9)
+    base = rng.uniform(1.0, 2.0, size=(8, 1000)).astype(np.float32)
+    base[0, 17] = np.nan
+    base[1, 500] = np.inf
+    base[2, 999] = -np.inf
+    base[3, :] = 1.5
+    base[4, 3] = -3.0e38
+    base[4, 4] = 3.0e38
+    base[5, :] = (rng.integers(0, 7, size=1000) * 1e-45).astype(np.float32)  # subnormals
+    base[6, :] = np.where(rng.random(1000) < 0.5, -0.0, 0.0).astype(np.float32)
+    base[7, :] = rng.uniform(-1e-30, 1e-30, size=1000).astype(np.float32)  # normal + subnormal, bucket path
+    host = np.ascontiguousarray(base).view(np.uint32)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+def test_bucket_tiny_and_huge_finite_ranges():
+    """range = 1 ulp (two distinct values) and range near FLT_MAX (finite)."""
+    one = np.float32(1.0)
+    up = np.nextafter(one, np.float32(2))
+    a = np.where(np.random.default_rng(1).random(1000) < 0.5, one, up).astype(np.float32)
+    b = np.random.default_rng(2).uniform(-1.6e38, 1.6e38, size=1000).astype(np.float32)
+    host = np.stack([a.view(np.uint32), b.view(np.uint32)])
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+def test_bucket_clustered_mixture_random():
+    """Clustered values: arrays randomly on either side of the capacity limit."""
+    rng = np.random.default_rng(11)
+    N = 2000
+    centers = rng.uniform(0, 100, size=(N, 3))
+    which = rng.integers(0, 3, size=(N, 1000))
+    widths = rng.choice([0.01, 0.3, 3.0, 30.0], size=(N, 1))
+    v = np.take_along_axis(centers, which, 1) + rng.normal(0, 1, size=(N, 1000)) * widths
+    host = np.ascontiguousarray(v.astype(np.float32)).view(np.uint32)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+def test_bucket_and_network_paths_agree(monkeypatch):
+    """GAS_BUCKET=0 (pure network) and the default give identical bits."""
+    host = datagen.fixed("paper_uniform", 7002, 0, 3000, 1000)
+    got_bucket = gpu_sort_fixed(host)
+    monkeypatch.setenv("GAS_BUCKET", "0")
+    got_net = gpu_sort_fixed(host)
+    np.testing.assert_array_equal(got_bucket, got_net)
+    np.testing.assert_array_equal(got_bucket, oracle_sorted(host))
