@@ -11,10 +11,11 @@
 // registers (6 compare-exchanges per key per bucket). Differences from the
 // paper, for B200: buckets come from linear interpolation between the array's
 // min and max (one FADD + one FFMA per key on the FMA pipe) instead of a
-// sorted sample and per-thread splitter scans (Alg. 1-2); ranks come from
-// conflict-free per-lane shared-memory counters and one rotated prefix scan
-// instead of a global bucket-size array Z (Def. 4); nothing but
-// the array itself touches HBM.
+// sorted sample and per-thread splitter scans (Alg. 1-2); a key's rank inside
+// its bucket comes from one shared-memory atomic increment of the bucket's
+// counter instead of a global bucket-size array Z (Def. 4), and
+// bucket starts from a warp scan of the 62 counts; nothing but the array
+// itself touches HBM.
 //
 // Correctness does not depend on the data: the bucket map
 //     b(v) = rn(rn(v - vmin) * s + 2^23) - 2^23,   s = rn(61 / rn(vmax - vmin))
@@ -44,20 +45,20 @@ constexpr int kBkBuckets = 62;  // value-interpolation buckets 0..61 (rows 62, 6
 #ifndef GAS_BK_WARPS_PER_SM
 #define GAS_BK_WARPS_PER_SM 16
 #endif
-#ifndef GAS_BK_PAIRCOUNT
-#define GAS_BK_PAIRCOUNT 1
+#ifndef GAS_BK_ATOMS
+#define GAS_BK_ATOMS 1  // ranks from shared atomics (1) or per-lane u16 counters + scan (0)
 #endif
 #ifndef GAS_BK_PREFETCH
 #define GAS_BK_PREFETCH 1
 #endif
 constexpr int kBkBlock = GAS_BK_BLOCK;
-// Per warp: u16 counters [64 rows (bucket)][32 lanes] (4 KB) — reused as the
-// position-order output staging buffer (n <= 1024 words) — then the slot
-// buffer [32 positions][64 buckets] of u32 keys (8 KB), also the 4 KB
-// transpose scratch of the fallback network.
-constexpr int kBkCntBytes = 64 * 32 * 2;
+// Per warp: 64 bucket counters (256 B), the slot buffer [32 positions][64
+// buckets] of u32 keys (8 KB; also the 4 KB transpose scratch of the fallback
+// network) and the position-order output staging buffer (n <= 1024 words).
+constexpr int kBkCntBytes = GAS_BK_ATOMS ? 64 * 4 : 64 * 32 * 2;
 constexpr int kBkSlotBytes = 32 * 64 * 4;
-constexpr int kBkWarpBytes = kBkCntBytes + kBkSlotBytes;
+constexpr int kBkOutBytes = 1024 * 4;
+constexpr int kBkWarpBytes = kBkCntBytes + kBkSlotBytes + kBkOutBytes;
 constexpr int kBkSmemBytes = (kBkBlock / 32) * kBkWarpBytes;
 
 __device__ __forceinline__ float fmin_nan(float a, float b) {
@@ -77,6 +78,11 @@ __device__ __forceinline__ uint32_t lds16(uint32_t a) {
 }
 __device__ __forceinline__ void sts16(uint32_t a, uint32_t v) {
   asm volatile("st.shared.u16 [%0], %1;" ::"r"(a), "h"((uint16_t)v) : "memory");
+}
+__device__ __forceinline__ uint32_t atoms_inc(uint32_t a) {
+  uint32_t v;
+  asm volatile("atom.shared.add.u32 %0, [%1], 1;" : "=r"(v) : "r"(a) : "memory");
+  return v;
 }
 __device__ __forceinline__ uint32_t lds32(uint32_t a) {
   uint32_t v;
@@ -103,8 +109,9 @@ __device__ __forceinline__ uint32_t bucket_bits(uint32_t raw, float vmin, float 
 }
 
 // The whole-array network (warp1024.cuh) for arrays the bucket map cannot
-// handle; out of line so that the bucket path's hot code stays compact.
-__device__ __noinline__ void bucket1024_fallback(uint32_t (&k)[32], uint4* dst, int nc, int lane, uint32_t* scratch,
+// handle. (Inline: an out-of-line call sends the key array through the stack
+// on every array, measured 84 local stores per array.)
+__device__ __forceinline__ void bucket1024_fallback(uint32_t (&k)[32], uint4* dst, int nc, int lane, uint32_t* scratch,
                                                  uint32_t one) {
   __syncwarp();
 #pragma unroll
@@ -131,13 +138,16 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
   extern __shared__ __align__(16) uint4 bk_smem[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
-  const uint32_t cnt_sa = wsa;                 // u16 counter (b, lane) at cnt_sa + b*64 + lane*2
-  const uint32_t slot_sa = wsa + kBkCntBytes;  // slot (p, b) at slot_sa + (p*64 + b)*4
+  const uint32_t cnt_sa = wsa;                                // counter of bucket b at cnt_sa + b*4
+  const uint32_t slot_sa = wsa + kBkCntBytes;                 // slot (p, b) at slot_sa + (p*64 + b)*4
+  const uint32_t out_sa = wsa + kBkCntBytes + kBkSlotBytes;   // output word p at out_sa + p*4
   uint32_t* const slot_ptr = reinterpret_cast<uint32_t*>(reinterpret_cast<unsigned char*>(bk_smem) +
                                                          warp * kBkWarpBytes + kBkCntBytes);
   const int nc = n >> 2;  // 16-byte chunks per array (> 128)
   const int64_t nwarps = (int64_t)gridDim.x * (kBkBlock / 32);
-  // counting address of bucket bits tb for this lane: cnt_sa + b*64 + lane*2
+  // counter address of bucket bits tb: tb*4 + cnt_b0
+  const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;
+  // (u16 counters) counter (b, lane) at cnt_sa + b*64 + lane*2 = tb*64 + cnt_lane0
   const uint32_t cnt_lane0 = cnt_sa + lane * 2 - 0x4B000000u * 64u;
   const uint32_t slot_b0 = slot_sa - 0x4B000000u * 4u;
 
@@ -180,26 +190,39 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     bool use_buckets = fabsf(vmin) <= 3.402823466e38f && fabsf(vmax) <= 3.402823466e38f && range > 0.0f &&
                        range <= 3.402823466e38f && s <= 3.402823466e38f;
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
-    uint32_t rk[32];
     if (use_buckets) {
-      // slot buffer <- pad keys, counters <- 0 (the previous array is done with both)
+#if GAS_BK_ATOMS
+      // bucket counters <- 0 (64 words; the previous array is done with them)
+      if (lane < 16) sts128(cnt_sa + lane * 16, make_uint4(0, 0, 0, 0));
+      __syncwarp();
+      // ---- rank: a shared-memory atomic increment of the key's bucket counter
+      // returns its rank inside the bucket (any order of equal-bucket keys is
+      // fine: the bucket is sorted afterwards)
+      uint32_t rk[32];
 #pragma unroll
-      for (int q = 0; q < kBkSlotBytes / 16 / 32; ++q)
-        sts128(slot_sa + (lane + 32 * q) * 16, make_uint4(kPadKey, kPadKey, kPadKey, kPadKey));
+      for (int r = 0; r < 32; ++r) {
+        const int q = r >> 2;
+        rk[r] = (q < 4 || lane + 32 * q < nc) ? atoms_inc(bucket_bits(k[r], vmin, s) * 4u + cnt_b0) : 0u;
+      }
+      __syncwarp();
+      t0 = lds32(cnt_sa + lane * 4);
+      t1 = lds32(cnt_sa + 128 + lane * 4);
+#else
+      // counters <- 0 (the previous array is done with them)
 #pragma unroll
       for (int q = 0; q < kBkCntBytes / 16 / 32; ++q) sts128(cnt_sa + (lane + 32 * q) * 16, make_uint4(0, 0, 0, 0));
       __syncwarp();
-      // ---- count: per-lane u16 counters, column `lane` of row b (conflict-free).
-      // Keys go in pairs so that the load -> increment -> store chain through
-      // shared memory has 16 links instead of 32: both counters are loaded
-      // first, and if both keys hit the same counter the second count is the
-      // first + 1 (the later store then leaves the right total).
+      // ---- count: per-lane u16 counters, column `lane` of row b. Keys go in
+      // pairs so that the load -> increment -> store chain through shared
+      // memory has 16 links instead of 32: both counters are loaded first, and
+      // if both keys hit the same counter the second count is the first + 1
+      // (the later store then leaves the right total).
+      uint32_t rk[32];
 #pragma unroll
       for (int r = 0; r < 32; r += 2) {
         const int q = r >> 2;
         if (q < 4 || lane + 32 * q < nc) {
           const uint32_t ca = bucket_bits(k[r], vmin, s) * 64u + cnt_lane0;
-#if GAS_BK_PAIRCOUNT
           const uint32_t cb = bucket_bits(k[r + 1], vmin, s) * 64u + cnt_lane0;
           const uint32_t c0 = lds16(ca);
           uint32_t c1 = lds16(cb);
@@ -208,15 +231,6 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
           sts16(cb, c1 + 1);
           rk[r] = c0;
           rk[r + 1] = c1;
-#else
-          const uint32_t c0 = lds16(ca);
-          sts16(ca, c0 + 1);
-          rk[r] = c0;
-          const uint32_t cb = bucket_bits(k[r + 1], vmin, s) * 64u + cnt_lane0;
-          const uint32_t c1 = lds16(cb);
-          sts16(cb, c1 + 1);
-          rk[r + 1] = c1;
-#endif
         } else {
           rk[r] = 0;
           rk[r + 1] = 0;
@@ -226,36 +240,45 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       // ---- scan: lane l turns rows l and l+32 into exclusive offsets. The
       // order of lanes inside a row is any fixed order (the chunks are read
       // rotated by lane/2 to avoid bank conflicts; lo halves before hi halves).
-      uint4 w[2][4];
+      {
+        uint4 w[2][4];
 #pragma unroll
-      for (int h = 0; h < 2; ++h)
+        for (int h = 0; h < 2; ++h)
 #pragma unroll
-        for (int q = 0; q < 4; ++q) w[h][q] = lds128(cnt_sa + (lane + 32 * h) * 64 + (((q + (lane >> 1)) & 3) << 4));
-      uint32_t tot[2];
+          for (int q = 0; q < 4; ++q) w[h][q] = lds128(cnt_sa + (lane + 32 * h) * 64 + (((q + (lane >> 1)) & 3) << 4));
+        uint32_t tot[2];
 #pragma unroll
-      for (int h = 0; h < 2; ++h) {
-        uint32_t sum = 0;
+        for (int h = 0; h < 2; ++h) {
+          uint32_t sum = 0;
 #pragma unroll
-        for (int q = 0; q < 4; ++q) sum += w[h][q].x + w[h][q].y + w[h][q].z + w[h][q].w;
-        const uint32_t tlo = sum & 0xFFFFu;
-        tot[h] = tlo + (sum >> 16);
-        uint32_t p = tlo << 16;
+          for (int q = 0; q < 4; ++q) sum += w[h][q].x + w[h][q].y + w[h][q].z + w[h][q].w;
+          const uint32_t tlo = sum & 0xFFFFu;
+          tot[h] = tlo + (sum >> 16);
+          uint32_t p = tlo << 16;
 #pragma unroll
-        for (int q = 0; q < 4; ++q) {
-          uint4 o;
-          o.x = p; p += w[h][q].x;
-          o.y = p; p += w[h][q].y;
-          o.z = p; p += w[h][q].z;
-          o.w = p; p += w[h][q].w;
-          w[h][q] = o;
+          for (int q = 0; q < 4; ++q) {
+            uint4 o;
+            o.x = p; p += w[h][q].x;
+            o.y = p; p += w[h][q].y;
+            o.z = p; p += w[h][q].z;
+            o.w = p; p += w[h][q].w;
+            w[h][q] = o;
+          }
         }
+#pragma unroll
+        for (int h = 0; h < 2; ++h)
+#pragma unroll
+          for (int q = 0; q < 4; ++q) sts128(cnt_sa + (lane + 32 * h) * 64 + (((q + (lane >> 1)) & 3) << 4), w[h][q]);
+        t0 = tot[0];
+        t1 = tot[1];
       }
+      __syncwarp();
 #pragma unroll
-      for (int h = 0; h < 2; ++h)
-#pragma unroll
-        for (int q = 0; q < 4; ++q) sts128(cnt_sa + (lane + 32 * h) * 64 + (((q + (lane >> 1)) & 3) << 4), w[h][q]);
-      t0 = tot[0];
-      t1 = tot[1];
+      for (int r = 0; r < 32; ++r) {
+        const int q = r >> 2;
+        if (q < 4 || lane + 32 * q < nc) rk[r] += lds16(bucket_bits(k[r], vmin, s) * 64u + cnt_lane0);
+      }
+#endif
       use_buckets = __all_sync(0xffffffffu, t0 <= 32u && t1 <= 32u);
       if (use_buckets) {
         // bucket bases: exclusive scan of the 64 bucket sizes (two 16-bit halves)
@@ -268,20 +291,12 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         const uint32_t total_lo = __shfl_sync(0xffffffffu, x & 0xFFFFu, 31);
         base0 = (x & 0xFFFFu) - t0;
         base1 = total_lo + (x >> 16) - t1;
-        __syncwarp();
         // ---- scatter: key of rank p in bucket b -> slot (p, b)
 #pragma unroll
         for (int r = 0; r < 32; ++r) {
           const int q = r >> 2;
-          if (q < 4 || lane + 32 * q < nc) rk[r] += lds16(bucket_bits(k[r], vmin, s) * 64u + cnt_lane0);
-        }
-#pragma unroll
-        for (int r = 0; r < 32; ++r) {
-          const int q = r >> 2;
-          if (q < 4 || lane + 32 * q < nc) {
-            const uint32_t sa = rk[r] * 256u + bucket_bits(k[r], vmin, s) * 4u + slot_b0;
-            sts32(sa, key_from_bits(k[r]));
-          }
+          if (q < 4 || lane + 32 * q < nc)
+            sts32(rk[r] * 256u + bucket_bits(k[r], vmin, s) * 4u + slot_b0, key_from_bits(k[r]));
         }
         __syncwarp();
       }
@@ -289,20 +304,19 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 
     if (use_buckets) {
       // ---- per round rho = 0, 1: gather bucket b = lane + 32 rho (its column
-      // of the slot buffer, conflict-free), sort it in registers, and stage its
-      // keys at output words base_b + i, i < size_b, in the dead counter region
-      // (4 KB = 1024 words >= n). Each staging store is predicated: stores of
-      // one lane to distinct addresses may be reordered, so no write may rely
-      // on another lane's later write. The round loop is rolled to keep the hot
-      // code inside the instruction cache.
-      const uint32_t out_sa = cnt_sa;
+      // of the slot buffer, conflict-free; slots i >= size_b are not read and
+      // hold the pad key), sort it in registers, and stage its keys at output
+      // words base_b + i, i < size_b. Each staging store is predicated: stores
+      // of one lane to distinct addresses may be reordered, so no write may
+      // rely on another lane's later write. The round loop is rolled to keep
+      // the hot code inside the instruction cache.
 #pragma unroll 1
       for (int rho = 0; rho < 2; ++rho) {
         const uint32_t col = slot_sa + lane * 4 + rho * 128;
         const uint32_t tb = rho ? t1 : t0;
         const uint32_t ob = out_sa + (rho ? base1 : base0) * 4;
 #pragma unroll
-        for (int i = 0; i < 32; ++i) k[i] = lds32(col + i * 256);
+        for (int i = 0; i < 32; ++i) k[i] = (uint32_t)i < tb ? lds32(col + i * 256) : kPadKey;
         sort32_regs(k, one);
 #pragma unroll
         for (int i = 0; i < 32; ++i)
