@@ -38,15 +38,17 @@
 
 namespace gas {
 
-constexpr int kBkBuckets = 62;  // value-interpolation buckets 0..61 (rows 62, 63 stay empty)
 #ifndef GAS_BK_BLOCK
 #define GAS_BK_BLOCK 128
 #endif
 #ifndef GAS_BK_WARPS_PER_SM
 #define GAS_BK_WARPS_PER_SM 16
 #endif
-#ifndef GAS_BK_ATOMS
-#define GAS_BK_ATOMS 1  // ranks from shared atomics (1) or per-lane u16 counters + scan (0)
+#ifndef GAS_BK_MIX_NUM  // compare-exchanges of the bucket networks in FMA form: NUM out of DEN
+#define GAS_BK_MIX_NUM 2
+#endif
+#ifndef GAS_BK_MIX_DEN
+#define GAS_BK_MIX_DEN 3
 #endif
 #ifndef GAS_BK_PREFETCH
 #define GAS_BK_PREFETCH 1
@@ -55,7 +57,7 @@ constexpr int kBkBlock = GAS_BK_BLOCK;
 // Per warp: 64 bucket counters (256 B), the slot buffer [32 positions][64
 // buckets] of u32 keys (8 KB; also the 4 KB transpose scratch of the fallback
 // network) and the position-order output staging buffer (n <= 1024 words).
-constexpr int kBkCntBytes = GAS_BK_ATOMS ? 64 * 4 : 64 * 32 * 2;
+constexpr int kBkCntBytes = 64 * 4;
 constexpr int kBkSlotBytes = 32 * 64 * 4;
 constexpr int kBkOutBytes = 1024 * 4;
 constexpr int kBkWarpBytes = kBkCntBytes + kBkSlotBytes + kBkOutBytes;
@@ -71,17 +73,12 @@ __device__ __forceinline__ float fmax_nan(float a, float b) {
   asm("max.NaN.f32 %0, %1, %2;" : "=f"(r) : "f"(a), "f"(b));
   return r;
 }
-__device__ __forceinline__ uint32_t lds16(uint32_t a) {
-  uint16_t v;
-  asm volatile("ld.shared.u16 %0, [%1];" : "=h"(v) : "r"(a) : "memory");
-  return v;
-}
-__device__ __forceinline__ void sts16(uint32_t a, uint32_t v) {
-  asm volatile("st.shared.u16 [%0], %1;" ::"r"(a), "h"((uint16_t)v) : "memory");
-}
-__device__ __forceinline__ uint32_t atoms_inc(uint32_t a) {
-  uint32_t v;
-  asm volatile("atom.shared.add.u32 %0, [%1], 1;" : "=r"(v) : "r"(a) : "memory");
+// Shared-memory accesses as ordered (volatile) PTX; the predicated forms
+// compile to one predicated instruction instead of a branch.
+__device__ __forceinline__ uint32_t atoms_inc_if(bool p, uint32_t a) {
+  uint32_t v = 0;
+  asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %1, 0;\n\t@q atom.shared.add.u32 %0, [%2], 1;\n\t}"
+               : "+r"(v) : "r"((uint32_t)p), "r"(a) : "memory");
   return v;
 }
 __device__ __forceinline__ uint32_t lds32(uint32_t a) {
@@ -91,6 +88,10 @@ __device__ __forceinline__ uint32_t lds32(uint32_t a) {
 }
 __device__ __forceinline__ void sts32(uint32_t a, uint32_t v) {
   asm volatile("st.shared.u32 [%0], %1;" ::"r"(a), "r"(v) : "memory");
+}
+__device__ __forceinline__ void sts32_if(bool p, uint32_t a, uint32_t v) {
+  asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %0, 0;\n\t@q st.shared.u32 [%1], %2;\n\t}"
+               ::"r"((uint32_t)p), "r"(a), "r"(v) : "memory");
 }
 __device__ __forceinline__ uint4 lds128(uint32_t a) {
   uint4 v;
@@ -108,11 +109,22 @@ __device__ __forceinline__ uint32_t bucket_bits(uint32_t raw, float vmin, float 
   return __float_as_uint(__fmaf_rn(dv, s, 8388608.0f));
 }
 
+// Batcher's 32-input odd-even merge sort in registers with this kernel's own
+// compare-exchange mix (bitonic.cuh ce<>).
+__device__ __forceinline__ void sort32_bk(uint32_t (&k)[32], uint32_t one) {
+  constexpr OddEvenTable<32> T{};
+#pragma unroll
+  for (int c = 0; c < OddEvenTable<32>::C; ++c) {
+    if ((c % GAS_BK_MIX_DEN) < GAS_BK_MIX_NUM) ce<true>(k[T.e[c].a], k[T.e[c].b], one);
+    else ce<false>(k[T.e[c].a], k[T.e[c].b], one);
+  }
+}
+
 // The whole-array network (warp1024.cuh) for arrays the bucket map cannot
 // handle. (Inline: an out-of-line call sends the key array through the stack
 // on every array, measured 84 local stores per array.)
 __device__ __forceinline__ void bucket1024_fallback(uint32_t (&k)[32], uint4* dst, int nc, int lane, uint32_t* scratch,
-                                                 uint32_t one) {
+                                                    uint32_t one) {
   __syncwarp();
 #pragma unroll
   for (int q = 0; q < 8; ++q) {
@@ -131,6 +143,22 @@ __device__ __forceinline__ void bucket1024_fallback(uint32_t (&k)[32], uint4* ds
   }
 }
 
+// Bucket round rho (0, 1) of one lane: gather bucket b = lane + 32 rho (its
+// column of the slot buffer, conflict-free; slots >= size_b hold the pad key),
+// sort it in registers and stage its keys at output words base_b + i, i <
+// size_b. Each staging store is predicated: stores of one lane to distinct
+// addresses may be reordered, so no write may rely on another lane's later
+// write. RAW: keys are raw float bits (all values > 0, unsigned order = value
+// order), else ordered keys (ordered_key.cuh).
+template <bool RAW>
+__device__ __forceinline__ void bucket_round(uint32_t (&k)[32], uint32_t col, uint32_t ob, uint32_t tb, uint32_t one) {
+#pragma unroll
+  for (int i = 0; i < 32; ++i) k[i] = lds32(col + i * 256);
+  sort32_bk(k, one);
+#pragma unroll
+  for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, RAW ? k[i] : bits_from_key(k[i]));
+}
+
 // Fixed-length arrays, 512 < n <= 1024, 16-byte-aligned rows (n % 4 == 0).
 // One warp per array (persistent grid-stride).
 __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
@@ -138,18 +166,15 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
   extern __shared__ __align__(16) uint4 bk_smem[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
-  const uint32_t cnt_sa = wsa;                                // counter of bucket b at cnt_sa + b*4
-  const uint32_t slot_sa = wsa + kBkCntBytes;                 // slot (p, b) at slot_sa + (p*64 + b)*4
-  const uint32_t out_sa = wsa + kBkCntBytes + kBkSlotBytes;   // output word p at out_sa + p*4
+  const uint32_t cnt_sa = wsa;                               // counter of bucket b at cnt_sa + b*4
+  const uint32_t slot_sa = wsa + kBkCntBytes;                // slot (p, b) at slot_sa + (p*64 + b)*4
+  const uint32_t out_sa = wsa + kBkCntBytes + kBkSlotBytes;  // output word p at out_sa + p*4
   uint32_t* const slot_ptr = reinterpret_cast<uint32_t*>(reinterpret_cast<unsigned char*>(bk_smem) +
                                                          warp * kBkWarpBytes + kBkCntBytes);
   const int nc = n >> 2;  // 16-byte chunks per array (> 128)
   const int64_t nwarps = (int64_t)gridDim.x * (kBkBlock / 32);
-  // counter address of bucket bits tb: tb*4 + cnt_b0
-  const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;
-  // (u16 counters) counter (b, lane) at cnt_sa + b*64 + lane*2 = tb*64 + cnt_lane0
-  const uint32_t cnt_lane0 = cnt_sa + lane * 2 - 0x4B000000u * 64u;
-  const uint32_t slot_b0 = slot_sa - 0x4B000000u * 4u;
+  const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;  // counter address = bucket bits * 4 + cnt_b0
+  constexpr uint32_t kSlotMinusCnt = kBkCntBytes;     // slot (0, b) address - counter b address
 
   for (int64_t a = (int64_t)blockIdx.x * (kBkBlock / 32) + warp; a < N; a += nwarps) {
     uint4* const dst = reinterpret_cast<uint4*>(d + a * (int64_t)n);
@@ -189,96 +214,30 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     // finite min and max (no NaN, no inf), distinct, finite range and scale
     bool use_buckets = fabsf(vmin) <= 3.402823466e38f && fabsf(vmax) <= 3.402823466e38f && range > 0.0f &&
                        range <= 3.402823466e38f && s <= 3.402823466e38f;
+    // every value > 0 (no zero of either sign, no negative): raw bits sort as unsigned
+    const bool raw = vmin > 0.0f;
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
     if (use_buckets) {
-#if GAS_BK_ATOMS
-      // bucket counters <- 0 (64 words; the previous array is done with them)
+      // slot buffer <- pad keys, bucket counters <- 0 (the previous array is done with both)
+#pragma unroll
+      for (int q = 0; q < kBkSlotBytes / 16 / 32; ++q)
+        sts128(slot_sa + (lane + 32 * q) * 16, make_uint4(kPadKey, kPadKey, kPadKey, kPadKey));
       if (lane < 16) sts128(cnt_sa + lane * 16, make_uint4(0, 0, 0, 0));
       __syncwarp();
       // ---- rank: a shared-memory atomic increment of the key's bucket counter
       // returns its rank inside the bucket (any order of equal-bucket keys is
-      // fine: the bucket is sorted afterwards)
-      uint32_t rk[32];
+      // fine: the bucket is sorted afterwards); the counter address is kept for
+      // the scatter (slot (p, b) = counter b + (p*64 + b)*4 - b*4 + const)
+      uint32_t rk[32], ca[32];
 #pragma unroll
       for (int r = 0; r < 32; ++r) {
         const int q = r >> 2;
-        rk[r] = (q < 4 || lane + 32 * q < nc) ? atoms_inc(bucket_bits(k[r], vmin, s) * 4u + cnt_b0) : 0u;
+        ca[r] = bucket_bits(k[r], vmin, s) * 4u + cnt_b0;
+        rk[r] = atoms_inc_if(q < 4 || lane + 32 * q < nc, ca[r]);
       }
       __syncwarp();
       t0 = lds32(cnt_sa + lane * 4);
       t1 = lds32(cnt_sa + 128 + lane * 4);
-#else
-      // counters <- 0 (the previous array is done with them)
-#pragma unroll
-      for (int q = 0; q < kBkCntBytes / 16 / 32; ++q) sts128(cnt_sa + (lane + 32 * q) * 16, make_uint4(0, 0, 0, 0));
-      __syncwarp();
-      // ---- count: per-lane u16 counters, column `lane` of row b. Keys go in
-      // pairs so that the load -> increment -> store chain through shared
-      // memory has 16 links instead of 32: both counters are loaded first, and
-      // if both keys hit the same counter the second count is the first + 1
-      // (the later store then leaves the right total).
-      uint32_t rk[32];
-#pragma unroll
-      for (int r = 0; r < 32; r += 2) {
-        const int q = r >> 2;
-        if (q < 4 || lane + 32 * q < nc) {
-          const uint32_t ca = bucket_bits(k[r], vmin, s) * 64u + cnt_lane0;
-          const uint32_t cb = bucket_bits(k[r + 1], vmin, s) * 64u + cnt_lane0;
-          const uint32_t c0 = lds16(ca);
-          uint32_t c1 = lds16(cb);
-          c1 = (ca == cb) ? c0 + 1 : c1;
-          sts16(ca, c0 + 1);
-          sts16(cb, c1 + 1);
-          rk[r] = c0;
-          rk[r + 1] = c1;
-        } else {
-          rk[r] = 0;
-          rk[r + 1] = 0;
-        }
-      }
-      __syncwarp();
-      // ---- scan: lane l turns rows l and l+32 into exclusive offsets. The
-      // order of lanes inside a row is any fixed order (the chunks are read
-      // rotated by lane/2 to avoid bank conflicts; lo halves before hi halves).
-      {
-        uint4 w[2][4];
-#pragma unroll
-        for (int h = 0; h < 2; ++h)
-#pragma unroll
-          for (int q = 0; q < 4; ++q) w[h][q] = lds128(cnt_sa + (lane + 32 * h) * 64 + (((q + (lane >> 1)) & 3) << 4));
-        uint32_t tot[2];
-#pragma unroll
-        for (int h = 0; h < 2; ++h) {
-          uint32_t sum = 0;
-#pragma unroll
-          for (int q = 0; q < 4; ++q) sum += w[h][q].x + w[h][q].y + w[h][q].z + w[h][q].w;
-          const uint32_t tlo = sum & 0xFFFFu;
-          tot[h] = tlo + (sum >> 16);
-          uint32_t p = tlo << 16;
-#pragma unroll
-          for (int q = 0; q < 4; ++q) {
-            uint4 o;
-            o.x = p; p += w[h][q].x;
-            o.y = p; p += w[h][q].y;
-            o.z = p; p += w[h][q].z;
-            o.w = p; p += w[h][q].w;
-            w[h][q] = o;
-          }
-        }
-#pragma unroll
-        for (int h = 0; h < 2; ++h)
-#pragma unroll
-          for (int q = 0; q < 4; ++q) sts128(cnt_sa + (lane + 32 * h) * 64 + (((q + (lane >> 1)) & 3) << 4), w[h][q]);
-        t0 = tot[0];
-        t1 = tot[1];
-      }
-      __syncwarp();
-#pragma unroll
-      for (int r = 0; r < 32; ++r) {
-        const int q = r >> 2;
-        if (q < 4 || lane + 32 * q < nc) rk[r] += lds16(bucket_bits(k[r], vmin, s) * 64u + cnt_lane0);
-      }
-#endif
       use_buckets = __all_sync(0xffffffffu, t0 <= 32u && t1 <= 32u);
       if (use_buckets) {
         // bucket bases: exclusive scan of the 64 bucket sizes (two 16-bit halves)
@@ -291,36 +250,32 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         const uint32_t total_lo = __shfl_sync(0xffffffffu, x & 0xFFFFu, 31);
         base0 = (x & 0xFFFFu) - t0;
         base1 = total_lo + (x >> 16) - t1;
-        // ---- scatter: key of rank p in bucket b -> slot (p, b)
+        // ---- scatter: key of rank p in bucket b -> slot (p, b); the slot
+        // address is the counter address ca = cnt_sa + b*4 moved by p*256 and
+        // by the fixed distance from the counters to column 0 of the slots
 #pragma unroll
         for (int r = 0; r < 32; ++r) {
           const int q = r >> 2;
-          if (q < 4 || lane + 32 * q < nc)
-            sts32(rk[r] * 256u + bucket_bits(k[r], vmin, s) * 4u + slot_b0, key_from_bits(k[r]));
+          const uint32_t sa = rk[r] * 256u + ca[r] + kSlotMinusCnt;
+          sts32_if(q < 4 || lane + 32 * q < nc, sa, raw ? k[r] : key_from_bits(k[r]));
         }
         __syncwarp();
       }
     }
 
     if (use_buckets) {
-      // ---- per round rho = 0, 1: gather bucket b = lane + 32 rho (its column
-      // of the slot buffer, conflict-free; slots i >= size_b are not read and
-      // hold the pad key), sort it in registers, and stage its keys at output
-      // words base_b + i, i < size_b. Each staging store is predicated: stores
-      // of one lane to distinct addresses may be reordered, so no write may
-      // rely on another lane's later write. The round loop is rolled to keep
-      // the hot code inside the instruction cache.
+      // ---- two bucket rounds per lane (rolled: the hot code stays in the
+      // instruction cache), then the coalesced in-place store
+      if (raw) {
 #pragma unroll 1
-      for (int rho = 0; rho < 2; ++rho) {
-        const uint32_t col = slot_sa + lane * 4 + rho * 128;
-        const uint32_t tb = rho ? t1 : t0;
-        const uint32_t ob = out_sa + (rho ? base1 : base0) * 4;
-#pragma unroll
-        for (int i = 0; i < 32; ++i) k[i] = (uint32_t)i < tb ? lds32(col + i * 256) : kPadKey;
-        sort32_regs(k, one);
-#pragma unroll
-        for (int i = 0; i < 32; ++i)
-          if ((uint32_t)i < tb) sts32(ob + i * 4, bits_from_key(k[i]));
+        for (int rho = 0; rho < 2; ++rho)
+          bucket_round<true>(k, slot_sa + lane * 4 + rho * 128, out_sa + (rho ? base1 : base0) * 4, rho ? t1 : t0,
+                             one);
+      } else {
+#pragma unroll 1
+        for (int rho = 0; rho < 2; ++rho)
+          bucket_round<false>(k, slot_sa + lane * 4 + rho * 128, out_sa + (rho ? base1 : base0) * 4, rho ? t1 : t0,
+                              one);
       }
       __syncwarp();
 #pragma unroll

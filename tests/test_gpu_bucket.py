@@ -132,3 +132,16 @@ def test_bucket_and_network_paths_agree(monkeypatch):
     got_net = gpu_sort_fixed(host)
     np.testing.assert_array_equal(got_bucket, got_net)
     np.testing.assert_array_equal(got_bucket, oracle_sorted(host))
+
+
+@pytest.mark.parametrize("lo,hi", [(-1000.0, 1000.0), (-5.0, -1e-3), (0.0, 1.0), (1e-3, 7.0)])
+def test_bucket_sign_modes(lo, hi):
+    """Mixed-sign and all-negative arrays (ordered-key path), arrays with zeros
+    (vmin = 0: ordered-key path) and all-positive arrays (raw-bit path)."""
+    rng = np.random.default_rng(int(abs(lo) * 7 + hi * 3))
+    v = rng.uniform(lo, hi, size=(600, 1000)).astype(np.float32)
+    if lo == 0.0:
+        v[:, ::97] = 0.0
+        v[::2, ::89] = -0.0
+    host = np.ascontiguousarray(v).view(np.uint32)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
