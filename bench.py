@@ -317,7 +317,10 @@ def main():
         pristine = torch.empty(N_rank, n, dtype=torch.float32, device=dev)
         datagen.fixed_device(pristine, dist, seed, i0, N_rank, n, stream.cuda_stream)
         alg_bytes = 8 * N_rank * n
-        kernel_hint = "k_fixed_warp" if n <= 1024 else "k_fixed_cta"
+        if 512 < n <= 1024 and n % 4 == 0 and os.environ.get("GAS_BUCKET", "1") != "0":
+            kernel_hint = "k_fixed_bucket1024"  # bucket-then-network kernel (aligned rows)
+        else:
+            kernel_hint = "k_fixed_warp" if n <= 1024 else "k_fixed_cta"
         n_desc = str(n)
     work = torch.empty_like(pristine)
 

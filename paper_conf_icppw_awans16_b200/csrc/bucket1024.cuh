@@ -54,13 +54,17 @@ namespace gas {
 #define GAS_BK_PREFETCH 1
 #endif
 constexpr int kBkBlock = GAS_BK_BLOCK;
-// Per warp: 64 bucket counters (256 B), the slot buffer [32 positions][64
-// buckets] of u32 keys (8 KB; also the 4 KB transpose scratch of the fallback
-// network) and the position-order output staging buffer (n <= 1024 words).
+// Per warp: 64 bucket counters (256 B), the slot buffer [64 buckets][36 words]
+// of u32 keys (9 KB; slot p of bucket b at word 36 b + p: the 36-word stride
+// makes both the random single-word scatter and the 16-byte row gathers of
+// 8 consecutive lanes spread over all banks; also the 4 KB transpose scratch
+// of the fallback network). Output word p is staged at word p of the slot
+// buffer: rows 0..31 (1152 words >= n) are free once round 0 has gathered
+// them, and round 1 reads only rows 32..63.
 constexpr int kBkCntBytes = 64 * 4;
-constexpr int kBkSlotBytes = 32 * 64 * 4;
-constexpr int kBkOutBytes = 1024 * 4;
-constexpr int kBkWarpBytes = kBkCntBytes + kBkSlotBytes + kBkOutBytes;
+constexpr int kBkRowWords = 36;  // slot row of one bucket: 32 slots + 4 words of skew
+constexpr int kBkSlotBytes = 64 * kBkRowWords * 4;
+constexpr int kBkWarpBytes = kBkCntBytes + kBkSlotBytes;
 constexpr int kBkSmemBytes = (kBkBlock / 32) * kBkWarpBytes;
 
 __device__ __forceinline__ float fmin_nan(float a, float b) {
@@ -144,16 +148,20 @@ __device__ __forceinline__ void bucket1024_fallback(uint32_t (&k)[32], uint4* ds
 }
 
 // Bucket round rho (0, 1) of one lane: gather bucket b = lane + 32 rho (its
-// column of the slot buffer, conflict-free; slots >= size_b hold the pad key),
+// slot row, 8 x 16 bytes, conflict-free; slots >= size_b hold the pad key),
 // sort it in registers and stage its keys at output words base_b + i, i <
 // size_b. Each staging store is predicated: stores of one lane to distinct
 // addresses may be reordered, so no write may rely on another lane's later
 // write. RAW: keys are raw float bits (all values > 0, unsigned order = value
 // order), else ordered keys (ordered_key.cuh).
 template <bool RAW>
-__device__ __forceinline__ void bucket_round(uint32_t (&k)[32], uint32_t col, uint32_t ob, uint32_t tb, uint32_t one) {
+__device__ __forceinline__ void bucket_round(uint32_t (&k)[32], uint32_t row, uint32_t ob, uint32_t tb, uint32_t one) {
 #pragma unroll
-  for (int i = 0; i < 32; ++i) k[i] = lds32(col + i * 256);
+  for (int q = 0; q < 8; ++q) {
+    const uint4 v = lds128(row + q * 16);
+    k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
+  }
+  __syncwarp();  // every lane has its row before any staging store can land on rows 0..31
   sort32_bk(k, one);
 #pragma unroll
   for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, RAW ? k[i] : bits_from_key(k[i]));
@@ -167,30 +175,27 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
   const uint32_t cnt_sa = wsa;                               // counter of bucket b at cnt_sa + b*4
-  const uint32_t slot_sa = wsa + kBkCntBytes;                // slot (p, b) at slot_sa + (p*64 + b)*4
-  const uint32_t out_sa = wsa + kBkCntBytes + kBkSlotBytes;  // output word p at out_sa + p*4
+  const uint32_t slot_sa = wsa + kBkCntBytes;                // slot (p, b) at slot_sa + (36 b + p)*4
+  const uint32_t out_sa = slot_sa;                           // output word p at out_sa + p*4 (rows 0..31)
   uint32_t* const slot_ptr = reinterpret_cast<uint32_t*>(reinterpret_cast<unsigned char*>(bk_smem) +
                                                          warp * kBkWarpBytes + kBkCntBytes);
   const int nc = n >> 2;  // 16-byte chunks per array (> 128)
   const int64_t nwarps = (int64_t)gridDim.x * (kBkBlock / 32);
   const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;  // counter address = bucket bits * 4 + cnt_b0
-  constexpr uint32_t kSlotMinusCnt = kBkCntBytes;     // slot (0, b) address - counter b address
+  // slot (p, b) address = 36 * (counter address of b) + 4 p + slot_c0
+  const uint32_t slot_c0 = slot_sa - (uint32_t)kBkRowWords * cnt_sa;
 
   for (int64_t a = (int64_t)blockIdx.x * (kBkBlock / 32) + warp; a < N; a += nwarps) {
     uint4* const dst = reinterpret_cast<uint4*>(d + a * (int64_t)n);
-    // ---- a2: stage in (raw bits). Pad slots repeat a real value of the lane
-    // (neutral for min/max) and are excluded from counting and scatter.
+    // ---- a2: stage in (raw bits). Slots past the end (only in chunks q >= 4,
+    // n > 512) are left out of min/max, counting and scatter.
     uint32_t k[32];
-    {
-      const uint4 v0 = ld_stream(dst + lane);
-      k[0] = v0.x; k[1] = v0.y; k[2] = v0.z; k[3] = v0.w;
 #pragma unroll
-      for (int q = 1; q < 8; ++q) {
-        const int c = lane + 32 * q;
-        uint4 v = make_uint4(v0.x, v0.x, v0.x, v0.x);
-        if (q < 4 || c < nc) v = ld_stream(dst + c);
-        k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
-      }
+    for (int q = 0; q < 8; ++q) {
+      const int c = lane + 32 * q;
+      uint4 v = make_uint4(0, 0, 0, 0);
+      if (q < 4 || c < nc) v = ld_stream(dst + c);
+      k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
     }
 #if GAS_BK_PREFETCH
     if (lane == 0 && a + nwarps < N)  // warm L2 with this warp's next array (one TMA bulk prefetch)
@@ -200,9 +205,19 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     // ---- bucket map parameters: min and max value (NaN-propagating)
     float vmin = __uint_as_float(k[0]), vmax = vmin;
 #pragma unroll
-    for (int r = 1; r < 32; ++r) {
+    for (int r = 1; r < 16; ++r) {
       vmin = fmin_nan(vmin, __uint_as_float(k[r]));
       vmax = fmax_nan(vmax, __uint_as_float(k[r]));
+    }
+#pragma unroll
+    for (int q = 4; q < 8; ++q) {
+      if (lane + 32 * q < nc) {
+#pragma unroll
+        for (int j = 0; j < 4; ++j) {
+          vmin = fmin_nan(vmin, __uint_as_float(k[4 * q + j]));
+          vmax = fmax_nan(vmax, __uint_as_float(k[4 * q + j]));
+        }
+      }
     }
 #pragma unroll
     for (int m = 16; m >= 1; m >>= 1) {
@@ -226,14 +241,12 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       __syncwarp();
       // ---- rank: a shared-memory atomic increment of the key's bucket counter
       // returns its rank inside the bucket (any order of equal-bucket keys is
-      // fine: the bucket is sorted afterwards); the counter address is kept for
-      // the scatter (slot (p, b) = counter b + (p*64 + b)*4 - b*4 + const)
-      uint32_t rk[32], ca[32];
+      // fine: the bucket is sorted afterwards)
+      uint32_t rk[32];
 #pragma unroll
       for (int r = 0; r < 32; ++r) {
         const int q = r >> 2;
-        ca[r] = bucket_bits(k[r], vmin, s) * 4u + cnt_b0;
-        rk[r] = atoms_inc_if(q < 4 || lane + 32 * q < nc, ca[r]);
+        rk[r] = atoms_inc_if(q < 4 || lane + 32 * q < nc, bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
       }
       __syncwarp();
       t0 = lds32(cnt_sa + lane * 4);
@@ -250,13 +263,13 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         const uint32_t total_lo = __shfl_sync(0xffffffffu, x & 0xFFFFu, 31);
         base0 = (x & 0xFFFFu) - t0;
         base1 = total_lo + (x >> 16) - t1;
-        // ---- scatter: key of rank p in bucket b -> slot (p, b); the slot
-        // address is the counter address ca = cnt_sa + b*4 moved by p*256 and
-        // by the fixed distance from the counters to column 0 of the slots
+        // ---- scatter: key of rank p in bucket b -> slot (p, b), addressed
+        // from the counter address ca = cnt_sa + 4 b
 #pragma unroll
         for (int r = 0; r < 32; ++r) {
           const int q = r >> 2;
-          const uint32_t sa = rk[r] * 256u + ca[r] + kSlotMinusCnt;
+          const uint32_t ca = bucket_bits(k[r], vmin, s) * 4u + cnt_b0;
+          const uint32_t sa = ca * (uint32_t)kBkRowWords + (rk[r] * 4u + slot_c0);
           sts32_if(q < 4 || lane + 32 * q < nc, sa, raw ? k[r] : key_from_bits(k[r]));
         }
         __syncwarp();
@@ -269,12 +282,12 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       if (raw) {
 #pragma unroll 1
         for (int rho = 0; rho < 2; ++rho)
-          bucket_round<true>(k, slot_sa + lane * 4 + rho * 128, out_sa + (rho ? base1 : base0) * 4, rho ? t1 : t0,
+          bucket_round<true>(k, slot_sa + (lane + 32 * rho) * (kBkRowWords * 4), out_sa + (rho ? base1 : base0) * 4, rho ? t1 : t0,
                              one);
       } else {
 #pragma unroll 1
         for (int rho = 0; rho < 2; ++rho)
-          bucket_round<false>(k, slot_sa + lane * 4 + rho * 128, out_sa + (rho ? base1 : base0) * 4, rho ? t1 : t0,
+          bucket_round<false>(k, slot_sa + (lane + 32 * rho) * (kBkRowWords * 4), out_sa + (rho ? base1 : base0) * 4, rho ? t1 : t0,
                               one);
       }
       __syncwarp();
