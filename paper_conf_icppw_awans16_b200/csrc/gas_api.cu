@@ -12,6 +12,7 @@
 #include "../../include/gas.h"
 #include "segsort.cuh"
 #include "bucket1024.cuh"
+#include "bucket_cta.cuh"
 #include "pairs.cuh"
 
 namespace {
@@ -79,10 +80,41 @@ cudaError_t launch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   return cudaGetLastError();
 }
 
+bool bucket_enabled() {
+  const char* v = std::getenv("GAS_BUCKET");
+  return !(v && std::strcmp(v, "0") == 0);
+}
+
+// Bucket-then-network, one array per CTA of W warps (bucket_cta.cuh).
+template <int W, bool VEC>
+cudaError_t launch_fixed_bucket_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  auto k = gas::k_fixed_bucket_cta<W, VEC>;
+  constexpr int smem = gas::BkCta<W>::SMEM;
+  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  if (e != cudaSuccess) return e;
+  k<<<persistent_grid_smem(k, 32 * W, smem, N), 32 * W, smem, s>>>(d, N, n, 1u);
+  return cudaGetLastError();
+}
+
+template <int W>
+cudaError_t launch_offsets_bucket(uint32_t* d, const int64_t* off, int64_t N, int64_t lo, int64_t hi,
+                                  unsigned long long* ctr, cudaStream_t s) {
+  auto k = gas::k_offsets_bucket<W>;
+  constexpr int smem = gas::BkCta<W>::SMEM;
+  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  if (e != cudaSuccess) return e;
+  k<<<persistent_grid_smem(k, 32 * W, smem, (N + 31) / 32), 32 * W, smem, s>>>(d, off, N, lo, hi, ctr, 1u);
+  return cudaGetLastError();
+}
+
 // Fixed-length CTA classes (n > 1024): W warps' network, WR = ceil(n / 1024) real
 // warps rounded to the instantiated set (padding blocks are virtual, see sort_cta).
 template <bool VEC>
 cudaError_t dispatch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  if (bucket_enabled() && n <= 4096) {
+    if (n <= 2048) return launch_fixed_bucket_cta<2, VEC>(d, N, n, s);
+    return launch_fixed_bucket_cta<4, VEC>(d, N, n, s);
+  }
   if (n <= 2048) return launch_fixed_cta<2, 2, VEC>(d, N, n, s);
   if (n <= 3072) return launch_fixed_cta<4, 3, VEC>(d, N, n, s);
   if (n <= 4096) return launch_fixed_cta<4, 4, VEC>(d, N, n, s);
@@ -125,11 +157,6 @@ cudaError_t launch_fixed_bucket1024(uint32_t* d, int64_t N, int n, cudaStream_t 
   return cudaGetLastError();
 }
 
-bool bucket_enabled() {
-  const char* v = std::getenv("GAS_BUCKET");
-  return !(v && std::strcmp(v, "0") == 0);
-}
-
 template <bool VEC>
 cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   switch (size_class(n)) {
@@ -148,6 +175,7 @@ cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
       // the kernel is ALU/issue-bound, not latency-bound.
       if (VEC && env_flag("GAS_TMA")) return launch_fixed_1024_tma(d, N, n, s);
       if (VEC && bucket_enabled()) return launch_fixed_bucket1024(d, N, n, s);
+      if (!VEC && bucket_enabled() && n > 512) return launch_fixed_bucket_cta<1, false>(d, N, n, s);
       return launch_fixed_warp<32, 32, VEC>(d, N, n, s);
     default: return dispatch_fixed_cta<VEC>(d, N, n, s);
   }
@@ -186,10 +214,18 @@ cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, i
     case 128: return launch_offsets_warp<32, 4>(d, off, N, s);
     case 256: return launch_offsets_warp<32, 8>(d, off, N, s);
     case 512: return launch_offsets_warp<32, 16>(d, off, N, s);
-    case 1024: return launch_offsets_warp<32, 32>(d, off, N, s);
-    case 2048: return launch_offsets_cta<2, 2>(d, off, N, 1024, 2048, ctr, s);
-    case 3072: return launch_offsets_cta<4, 3>(d, off, N, 2048, 3072, ctr + 1, s);
-    case 4096: return launch_offsets_cta<4, 4>(d, off, N, 3072, 4096, ctr + 2, s);
+    case 1024:
+      if (bucket_enabled()) return launch_offsets_bucket<1>(d, off, N, 512, 1024, ctr + 7, s);
+      return launch_offsets_warp<32, 32>(d, off, N, s);
+    case 2048:
+      if (bucket_enabled()) return launch_offsets_bucket<2>(d, off, N, 1024, 2048, ctr, s);
+      return launch_offsets_cta<2, 2>(d, off, N, 1024, 2048, ctr, s);
+    case 3072:
+      if (bucket_enabled()) return launch_offsets_bucket<4>(d, off, N, 2048, 3072, ctr + 1, s);
+      return launch_offsets_cta<4, 3>(d, off, N, 2048, 3072, ctr + 1, s);
+    case 4096:
+      if (bucket_enabled()) return launch_offsets_bucket<4>(d, off, N, 3072, 4096, ctr + 2, s);
+      return launch_offsets_cta<4, 4>(d, off, N, 3072, 4096, ctr + 2, s);
     case 6144: return launch_offsets_cta<8, 6>(d, off, N, 4096, 6144, ctr + 3, s);
     case 8192: return launch_offsets_cta<8, 8>(d, off, N, 6144, 8192, ctr + 4, s);
     case 12288: return launch_offsets_cta<16, 12>(d, off, N, 8192, 12288, ctr + 5, s);
@@ -268,7 +304,7 @@ struct HostStaging {
 HostStaging g_staging[kMaxDevices];
 
 // Per-(device, stream) window counters of the offsets variant (see there).
-constexpr int kCounters = 7;
+constexpr int kCounters = 8;
 std::mutex g_ctr_mu;
 std::map<std::pair<int, cudaStream_t>, unsigned long long*> g_ctr;
 
@@ -332,11 +368,11 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
     if (h) return GAS_ERROR_INVALID_VALUE;
   }
   uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
-  // 7 window counters for the CTA classes' dynamic scheduling: 56 bytes per
+  // 8 window counters for the CTA classes' dynamic scheduling: 64 bytes per
   // (device, stream), allocated on first use and re-zeroed in stream order by
   // every call (calls on one stream are ordered; different streams never share)
   unsigned long long* ctr = nullptr;
-  if (max_array_len > 1024) {
+  if (max_array_len > 512) {
     cudaError_t e = counters_for(stream, &ctr);
     if (e == cudaSuccess) e = cudaMemsetAsync(ctr, 0, kCounters * sizeof(unsigned long long), stream);
     if (e != cudaSuccess) return cuda_fail(e);

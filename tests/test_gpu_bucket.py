@@ -145,3 +145,70 @@ def test_bucket_sign_modes(lo, hi):
         v[::2, ::89] = -0.0
     host = np.ascontiguousarray(v).view(np.uint32)
     np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+# ---- CTA bucket kernels (bucket_cta.cuh): W = 1 (unaligned n <= 1024), 2, 4
+
+from tests.test_gpu_parity import gpu_sort_offsets  # noqa: E402
+
+
+@pytest.mark.parametrize("n", [1025, 1500, 2000, 2048, 2049, 3000, 3072, 3073, 4000, 4096])
+@pytest.mark.parametrize("dist", ["paper_uniform", "spectra_mz", "sorted", "special_mix", "dup16"])
+def test_bucket_cta_fixed(dist, n):
+    host = datagen.fixed(dist, 7101, 0, 150, n)
+    expect = oracle_sorted(host)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=4), expect)  # 16-byte rows when n % 4 == 0
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=1), expect)  # scalar path
+
+
+@pytest.mark.parametrize("n", [513, 700, 999, 1000, 1024])
+@pytest.mark.parametrize("dist", ["paper_uniform", "reverse", "special_mix"])
+def test_bucket_cta_unaligned_warp_class(dist, n):
+    host = datagen.fixed(dist, 7102, 0, 400, n)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=3), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("count", [32, 33])
+def test_bucket_cta_capacity_edge(count):
+    """n = 4000 (W = 4, 248 buckets): vmin = 0, vmax = 247 maps b(v) = rint(v)."""
+    rng = np.random.default_rng(100 + count)
+    rows = []
+    for i in range(16):
+        vals = [0.0, 247.0] + list(100.0 + rng.uniform(-0.49, 0.49, size=count))
+        rest = 4000 - len(vals)
+        others = [b for b in range(1, 247) if b != 100]
+        per = np.bincount(np.arange(rest) % len(others), minlength=len(others))
+        for b, c in zip(others, per):
+            vals += list(b + rng.uniform(-0.45, 0.45, size=c))
+        v = np.array(vals, dtype=np.float32)
+        rng.shuffle(v)
+        rows.append(v.view(np.uint32))
+    host = np.stack(rows)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=4), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("dist", ["paper_uniform", "spectra_mz", "sorted", "special_mix", "spectra_intensity"])
+def test_bucket_offsets_classes(dist):
+    """Variable lengths through the 1024 / 2048 / 3072 / 4096 bucket classes,
+    every start alignment."""
+    lens = datagen.lengths(7103, 0, 2500, 400, 4096)
+    lens[:6] = [513, 1024, 1025, 2048, 3073, 4096]
+    off = datagen.offsets_from_lengths(lens)
+    data = datagen.ragged(dist, 7103, 0, off)
+    expect = data.copy()
+    oracle.sort_arrays_offsets_(expect, off)
+    for lead in (0, 1, 3):
+        np.testing.assert_array_equal(gpu_sort_offsets(data, off, lead=lead), expect)
+
+
+def test_bucket_offsets_mixed_signs_and_network_agree(monkeypatch):
+    rng = np.random.default_rng(7104)
+    lens = rng.integers(513, 4097, size=1500)
+    off = datagen.offsets_from_lengths(lens)
+    data = rng.uniform(-50, 50, size=int(off[-1])).astype(np.float32).view(np.uint32)
+    expect = data.copy()
+    oracle.sort_arrays_offsets_(expect, off)
+    got = gpu_sort_offsets(data, off, lead=2)
+    np.testing.assert_array_equal(got, expect)
+    monkeypatch.setenv("GAS_BUCKET", "0")
+    np.testing.assert_array_equal(gpu_sort_offsets(data, off, lead=2), expect)
