@@ -58,13 +58,14 @@ constexpr int kBkBlock = GAS_BK_BLOCK;
 // of u32 keys (9 KB; slot p of bucket b at word 36 b + p: the 36-word stride
 // makes both the random single-word scatter and the 16-byte row gathers of
 // 8 consecutive lanes spread over all banks; also the 4 KB transpose scratch
-// of the fallback network). Output word p is staged at word p of the slot
-// buffer: rows 0..31 (1152 words >= n) are free once round 0 has gathered
-// them, and round 1 reads only rows 32..63.
+// of the fallback network), and a separate 4 KB output staging buffer (output
+// word p at word p; the rounds run buckets 32..63 first, so rows 0..31 are
+// still live while the first round stages its output).
 constexpr int kBkCntBytes = 64 * 4;
 constexpr int kBkRowWords = 36;  // slot row of one bucket: 32 slots + 4 words of skew
 constexpr int kBkSlotBytes = 64 * kBkRowWords * 4;
-constexpr int kBkWarpBytes = kBkCntBytes + kBkSlotBytes;
+constexpr int kBkOutBytes = 1024 * 4;
+constexpr int kBkWarpBytes = kBkCntBytes + kBkSlotBytes + kBkOutBytes;
 constexpr int kBkSmemBytes = (kBkBlock / 32) * kBkWarpBytes;
 
 __device__ __forceinline__ float fmin_nan(float a, float b) {
@@ -147,28 +148,51 @@ __device__ __forceinline__ void bucket1024_fallback(uint32_t (&k)[32], uint4* ds
   }
 }
 
-// Bucket round rho (0, 1) of one lane: gather bucket b = lane + 32 rho (its
-// slot row, 8 x 16 bytes, conflict-free; slots >= size_b hold the pad key),
-// sort it in registers and stage its keys at output words base_b + i, i <
-// size_b. Each staging store is predicated: stores of one lane to distinct
-// addresses may be reordered, so no write may rely on another lane's later
-// write. RAW: keys are raw float bits (all values > 0, unsigned order = value
-// order), else ordered keys (ordered_key.cuh).
-template <bool RAW>
-__device__ __forceinline__ void bucket_round(uint32_t (&k)[32], uint32_t row, uint32_t ob, uint32_t tb, uint32_t one) {
-#pragma unroll
-  for (int q = 0; q < 8; ++q) {
-    const uint4 v = lds128(row + q * 16);
-    k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
-  }
-  __syncwarp();  // every lane has its row before any staging store can land on rows 0..31
-  sort32_bk(k, one);
-#pragma unroll
-  for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, RAW ? k[i] : bits_from_key(k[i]));
+
+// Predicated forms of the global / shared accesses of the kernel below (one
+// predicated instruction each instead of a branch around it).
+__device__ __forceinline__ uint4 ldg_cs_if(bool p, const uint4* a) {
+  uint4 v = make_uint4(0, 0, 0, 0);
+  asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %4, 0;\n\t@q ld.global.cs.v4.u32 {%0, %1, %2, %3}, [%5];\n\t}"
+               : "+r"(v.x), "+r"(v.y), "+r"(v.z), "+r"(v.w) : "r"((uint32_t)p), "l"(a) : "memory");
+  return v;
+}
+__device__ __forceinline__ void stg_cs_if(bool p, uint4* a, uint4 v) {
+  asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %0, 0;\n\t@q st.global.cs.v4.u32 [%1], {%2, %3, %4, %5};\n\t}"
+               ::"r"((uint32_t)p), "l"(a), "r"(v.x), "r"(v.y), "r"(v.z), "r"(v.w) : "memory");
+}
+// Loads the 16-byte chunk at shared address a into x..w when p; else leaves them.
+__device__ __forceinline__ void lds128_if(bool p, uint32_t a, uint32_t& x, uint32_t& y, uint32_t& z, uint32_t& w) {
+  asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %4, 0;\n\t@q ld.shared.v4.u32 {%0, %1, %2, %3}, [%5];\n\t}"
+               : "+r"(x), "+r"(y), "+r"(z), "+r"(w) : "r"((uint32_t)p), "r"(a) : "memory");
+}
+// Atomic add of 4 to the shared word at a, returning the old value (0 when !p).
+__device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
+  uint32_t v = 0;
+  asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %1, 0;\n\t@q atom.shared.add.u32 %0, [%2], 4;\n\t}"
+               : "+r"(v) : "r"((uint32_t)p), "r"(a) : "memory");
+  return v;
 }
 
 // Fixed-length arrays, 512 < n <= 1024, 16-byte-aligned rows (n % 4 == 0).
-// One warp per array (persistent grid-stride).
+// One warp per array (persistent grid-stride). Per array:
+//  1. load (8 x LDG.128 per lane); min / max of the raw bits (VIMNMX3 + REDUX).
+//     All values positive and finite (the paper's data): the raw
+//     bits sort as unsigned integers and are the keys ("raw" arrays); else the
+//     keys are the totalOrder transform (ordered_key.cuh) and an infinity or
+//     NaN sends the array to the fallback network.
+//  2. bucket counter b starts at the shared address of slot 0 of bucket row b
+//     and each key adds 4 to it: the atomic's old value IS the key's slot
+//     address (bucket row b, rank = arrival order).
+//  3. one store of 16 pad bytes at the row's first chunk past its keys, then
+//     the scatter (one store per key).
+//  4. rounds: lane l sorts bucket l + 32 first, then bucket l. Only the
+//     ceil(size/4) chunks holding keys are gathered: the other registers hold
+//     pads (first round) or the sorted keys of bucket l + 32 (second round),
+//     which all follow every key of bucket l (the map is monotone), so the
+//     first size_b network outputs are bucket b sorted in both rounds.
+//     Outputs are staged at words base_b + i of the output buffer.
+//  5. coalesced in-place store (key -> bits for non-raw arrays).
 __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     k_fixed_bucket1024(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   extern __shared__ __align__(16) uint4 bk_smem[];
@@ -176,25 +200,24 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
   const uint32_t cnt_sa = wsa;                               // counter of bucket b at cnt_sa + b*4
   const uint32_t slot_sa = wsa + kBkCntBytes;                // slot (p, b) at slot_sa + (36 b + p)*4
-  const uint32_t out_sa = slot_sa;                           // output word p at out_sa + p*4 (rows 0..31)
+  const uint32_t out_sa = slot_sa + kBkSlotBytes;            // output word p at out_sa + p*4
   uint32_t* const slot_ptr = reinterpret_cast<uint32_t*>(reinterpret_cast<unsigned char*>(bk_smem) +
                                                          warp * kBkWarpBytes + kBkCntBytes);
   const int nc = n >> 2;  // 16-byte chunks per array (> 128)
   const int64_t nwarps = (int64_t)gridDim.x * (kBkBlock / 32);
   const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;  // counter address = bucket bits * 4 + cnt_b0
-  // slot (p, b) address = 36 * (counter address of b) + 4 p + slot_c0
-  const uint32_t slot_c0 = slot_sa - (uint32_t)kBkRowWords * cnt_sa;
+  const uint32_t row0 = slot_sa + lane * (kBkRowWords * 4);  // this lane's rows: buckets lane, lane + 32
+  const uint32_t row1 = row0 + 32 * (kBkRowWords * 4);
+  const uint4 pad4 = make_uint4(kPadKey, kPadKey, kPadKey, kPadKey);
 
   for (int64_t a = (int64_t)blockIdx.x * (kBkBlock / 32) + warp; a < N; a += nwarps) {
     uint4* const dst = reinterpret_cast<uint4*>(d + a * (int64_t)n);
-    // ---- a2: stage in (raw bits). Slots past the end (only in chunks q >= 4,
-    // n > 512) are left out of min/max, counting and scatter.
+    // ---- a2: stage in (raw bits); chunks q >= 4 may lie past the end (n > 512)
     uint32_t k[32];
 #pragma unroll
     for (int q = 0; q < 8; ++q) {
       const int c = lane + 32 * q;
-      uint4 v = make_uint4(0, 0, 0, 0);
-      if (q < 4 || c < nc) v = ld_stream(dst + c);
+      const uint4 v = q < 4 ? ld_stream(dst + c) : ldg_cs_if(c < nc, dst + c);
       k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
     }
 #if GAS_BK_PREFETCH
@@ -202,55 +225,55 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + (a + nwarps) * (int64_t)n),
                    "r"((uint32_t)n * 4u) : "memory");
 #endif
-    // ---- bucket map parameters: min and max value (NaN-propagating)
-    float vmin = __uint_as_float(k[0]), vmax = vmin;
-#pragma unroll
-    for (int r = 1; r < 16; ++r) {
-      vmin = fmin_nan(vmin, __uint_as_float(k[r]));
-      vmax = fmax_nan(vmax, __uint_as_float(k[r]));
-    }
+    // slots past the end repeat k[0] so that min / max need no predicates
 #pragma unroll
     for (int q = 4; q < 8; ++q) {
-      if (lane + 32 * q < nc) {
+      const bool v = lane + 32 * q < nc;
 #pragma unroll
-        for (int j = 0; j < 4; ++j) {
-          vmin = fmin_nan(vmin, __uint_as_float(k[4 * q + j]));
-          vmax = fmax_nan(vmax, __uint_as_float(k[4 * q + j]));
-        }
-      }
+      for (int j = 0; j < 4; ++j) k[4 * q + j] = v ? k[4 * q + j] : k[0];
     }
+    // ---- bucket map parameters
+    uint32_t umin = k[0], umax = k[0];
 #pragma unroll
-    for (int m = 16; m >= 1; m >>= 1) {
-      vmin = fmin_nan(vmin, __shfl_xor_sync(0xffffffffu, vmin, m));
-      vmax = fmax_nan(vmax, __shfl_xor_sync(0xffffffffu, vmax, m));
+    for (int r = 1; r < 31; r += 2) {
+      umin = __vimin3_u32(umin, k[r], k[r + 1]);
+      umax = __vimax3_u32(umax, k[r], k[r + 1]);
     }
-    const float range = __fsub_rn(vmax, vmin);
-    const float s = __fdiv_rn(61.0f, range);
-    // finite min and max (no NaN, no inf), distinct, finite range and scale
-    bool use_buckets = fabsf(vmin) <= 3.402823466e38f && fabsf(vmax) <= 3.402823466e38f && range > 0.0f &&
-                       range <= 3.402823466e38f && s <= 3.402823466e38f;
-    // every value > 0 (no zero of either sign, no negative): raw bits sort as unsigned
-    const bool raw = vmin > 0.0f;
-    uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
-    if (use_buckets) {
-      // slot buffer <- pad keys, bucket counters <- 0 (the previous array is done with both)
-#pragma unroll
-      for (int q = 0; q < kBkSlotBytes / 16 / 32; ++q)
-        sts128(slot_sa + (lane + 32 * q) * 16, make_uint4(kPadKey, kPadKey, kPadKey, kPadKey));
-      if (lane < 16) sts128(cnt_sa + lane * 16, make_uint4(0, 0, 0, 0));
-      __syncwarp();
-      // ---- rank: a shared-memory atomic increment of the key's bucket counter
-      // returns its rank inside the bucket (any order of equal-bucket keys is
-      // fine: the bucket is sorted afterwards)
-      uint32_t rk[32];
+    umin = __reduce_min_sync(0xffffffffu, min(umin, k[31]));
+    umax = __reduce_max_sync(0xffffffffu, max(umax, k[31]));
+    const bool raw = umin > 0u && umax < 0x7F800000u;  // every value positive and finite
+    bool use_buckets = true;
+    if (!raw) {  // min / max in key space; an infinity or NaN (either sign) -> fallback
+      uint32_t kmin = 0xFFFFFFFFu, kmax = 0u;
 #pragma unroll
       for (int r = 0; r < 32; ++r) {
-        const int q = r >> 2;
-        rk[r] = atoms_inc_if(q < 4 || lane + 32 * q < nc, bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+        const uint32_t kk = key_from_bits(k[r]);
+        kmin = min(kmin, kk);
+        kmax = max(kmax, kk);
       }
+      kmin = __reduce_min_sync(0xffffffffu, kmin);
+      kmax = __reduce_max_sync(0xffffffffu, kmax);
+      use_buckets = kmin > 0x007FFFFFu && kmax < 0xFF800000u;
+      umin = bits_from_key(kmin);
+      umax = bits_from_key(kmax);
+    }
+    const float vmin = __uint_as_float(umin), vmax = __uint_as_float(umax);
+    const float range = __fsub_rn(vmax, vmin);
+    const float s = __fdiv_rn(61.0f, range);
+    use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
+    uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
+    if (use_buckets) {
+      sts32(cnt_sa + lane * 4, row0);
+      sts32(cnt_sa + 128 + lane * 4, row1);
       __syncwarp();
-      t0 = lds32(cnt_sa + lane * 4);
-      t1 = lds32(cnt_sa + 128 + lane * 4);
+      // ---- rank: the atomic returns the key's slot address
+      uint32_t sa[32];
+#pragma unroll
+      for (int r = 0; r < 32; ++r)
+        sa[r] = atoms_add4_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+      __syncwarp();
+      t0 = (lds32(cnt_sa + lane * 4) - row0) >> 2;
+      t1 = (lds32(cnt_sa + 128 + lane * 4) - row1) >> 2;
       use_buckets = __all_sync(0xffffffffu, t0 <= 32u && t1 <= 32u);
       if (use_buckets) {
         // bucket bases: exclusive scan of the 64 bucket sizes (two 16-bit halves)
@@ -263,14 +286,17 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         const uint32_t total_lo = __shfl_sync(0xffffffffu, x & 0xFFFFu, 31);
         base0 = (x & 0xFFFFu) - t0;
         base1 = total_lo + (x >> 16) - t1;
-        // ---- scatter: key of rank p in bucket b -> slot (p, b), addressed
-        // from the counter address ca = cnt_sa + 4 b
+        // pads after the last key of each row (t <= 32: chunk 8 is the row's skew)
+        sts128(row0 + (t0 >> 2) * 16, pad4);
+        sts128(row1 + (t1 >> 2) * 16, pad4);
+        __syncwarp();
+        // ---- scatter
+        if (raw) {
 #pragma unroll
-        for (int r = 0; r < 32; ++r) {
-          const int q = r >> 2;
-          const uint32_t ca = bucket_bits(k[r], vmin, s) * 4u + cnt_b0;
-          const uint32_t sa = ca * (uint32_t)kBkRowWords + (rk[r] * 4u + slot_c0);
-          sts32_if(q < 4 || lane + 32 * q < nc, sa, raw ? k[r] : key_from_bits(k[r]));
+          for (int r = 0; r < 32; ++r) sts32_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, sa[r], k[r]);
+        } else {
+#pragma unroll
+          for (int r = 0; r < 32; ++r) sts32_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, sa[r], key_from_bits(k[r]));
         }
         __syncwarp();
       }
@@ -278,23 +304,37 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 
     if (use_buckets) {
       // ---- two bucket rounds per lane (rolled: the hot code stays in the
-      // instruction cache), then the coalesced in-place store
-      if (raw) {
+      // instruction cache): bucket lane + 32, then bucket lane
 #pragma unroll 1
-        for (int rho = 0; rho < 2; ++rho)
-          bucket_round<true>(k, slot_sa + (lane + 32 * rho) * (kBkRowWords * 4), out_sa + (rho ? base1 : base0) * 4, rho ? t1 : t0,
-                             one);
-      } else {
-#pragma unroll 1
-        for (int rho = 0; rho < 2; ++rho)
-          bucket_round<false>(k, slot_sa + (lane + 32 * rho) * (kBkRowWords * 4), out_sa + (rho ? base1 : base0) * 4, rho ? t1 : t0,
-                              one);
+      for (int rho = 0; rho < 2; ++rho) {
+        const uint32_t tb = rho ? t0 : t1;
+        const uint32_t row = rho ? row0 : row1;
+        const uint32_t ob = out_sa + (rho ? base0 : base1) * 4;
+        if (rho == 0) {
+#pragma unroll
+          for (int i = 0; i < 32; ++i) k[i] = kPadKey;
+        }
+#pragma unroll
+        for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
+        sort32_bk(k, one);
+#pragma unroll
+        for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
       }
       __syncwarp();
+      if (raw) {
 #pragma unroll
-      for (int q = 0; q < 8; ++q) {
-        const int c = lane + 32 * q;
-        if (c < nc) st_stream(dst + c, lds128(out_sa + c * 16));
+        for (int q = 0; q < 8; ++q) {
+          const int c = lane + 32 * q;
+          stg_cs_if(q < 4 || c < nc, dst + c, lds128(out_sa + c * 16));
+        }
+      } else {
+#pragma unroll
+        for (int q = 0; q < 8; ++q) {
+          const int c = lane + 32 * q;
+          uint4 v = lds128(out_sa + c * 16);
+          v.x = bits_from_key(v.x); v.y = bits_from_key(v.y); v.z = bits_from_key(v.z); v.w = bits_from_key(v.w);
+          stg_cs_if(q < 4 || c < nc, dst + c, v);
+        }
       }
     } else {
       bucket1024_fallback(k, dst, nc, lane, slot_ptr, one);
