@@ -4,7 +4,7 @@
 // Why: the pure sorting network of warp1024.cuh spends ~26 compare-exchanges
 // per key (levels 6-10 of a 1024-key merge network) and is bound by the
 // integer-ALU pipe and instruction issue. This kernel first
-// splits the array into 62 value ranges — the paper's own idea of
+// splits the array into 64 value ranges — the paper's own idea of
 // data-independent buckets whose concatenation is the sorted array with no
 // merge step (§4.1, Alg. 2 P:L250-297 §5.2) — and then sorts each
 // bucket (<= 32 keys) with the 191-comparator odd-even network in one lane's
@@ -14,16 +14,17 @@
 // sorted sample and per-thread splitter scans (Alg. 1-2); a key's rank inside
 // its bucket comes from one shared-memory atomic increment of the bucket's
 // counter instead of a global bucket-size array Z (Def. 4), and
-// bucket starts from a warp scan of the 62 counts; nothing but the array
+// bucket starts from a warp scan of the 64 counts; nothing but the array
 // itself touches HBM.
 //
 // Correctness does not depend on the data: the bucket map
-//     b(v) = rn(rn(v - vmin) * s + 2^23) - 2^23,   s = rn(61 / rn(vmax - vmin))
+//     b(v) = rn(rn(v - vmin) * s + 2^23) - 2^23,   s = rn(TOP / rn(vmax - vmin))
 // is monotone non-decreasing in v (every step is a monotone rounding of a
 // monotone function), so every key of bucket b precedes (in IEEE totalOrder,
 // DESIGN.md reading C-1) every key of bucket b+1, and ±0 (equal values) share
-// a bucket whose network orders them. 0 <= b <= 61 because rn(v - vmin) lies
-// in [0, rn(vmax - vmin)] and range * s <= 61 (1 + 2^-24) < 61.5.
+// a bucket whose network orders them. 0 <= b <= TOP because rn(v - vmin) lies
+// in [0, rn(vmax - vmin)] and range * s <= TOP (1 + 2^-24) < TOP + 1/2
+// (TOP = GAS_BK_TOP = 63 for the warp kernel: 64 buckets; 61 W in bucket_cta.cuh).
 // The warp falls back to the full network (warp1024.cuh) for the whole array
 // when the map cannot be used — a NaN or an infinity in the array, all values
 // equal, a range that overflows or underflows — or when a bucket would hold
@@ -42,7 +43,7 @@ namespace gas {
 #define GAS_BK_BLOCK 128
 #endif
 #ifndef GAS_BK_WARPS_PER_SM
-#define GAS_BK_WARPS_PER_SM 16
+#define GAS_BK_WARPS_PER_SM 20
 #endif
 #ifndef GAS_BK_MIX_NUM  // compare-exchanges of the bucket networks in FMA form: NUM out of DEN
 #define GAS_BK_MIX_NUM 2
@@ -50,22 +51,29 @@ namespace gas {
 #ifndef GAS_BK_MIX_DEN
 #define GAS_BK_MIX_DEN 3
 #endif
+#ifndef GAS_BK_TOP  // the fixed-length warp kernel's buckets are 0 .. GAS_BK_TOP (<= 63)
+#define GAS_BK_TOP 63
+#endif
+#ifndef GAS_BK_TIERS  // network sizes per bucket round: 1 = always 32; 2 = 28 or 32; 3 = 24, 28 or 32
+#define GAS_BK_TIERS 1
+#endif
 #ifndef GAS_BK_PREFETCH
 #define GAS_BK_PREFETCH 1
 #endif
 constexpr int kBkBlock = GAS_BK_BLOCK;
-// Per warp: 64 bucket counters (256 B), the slot buffer [64 buckets][36 words]
-// of u32 keys (9 KB; slot p of bucket b at word 36 b + p: the 36-word stride
-// makes both the random single-word scatter and the 16-byte row gathers of
-// 8 consecutive lanes spread over all banks; also the 4 KB transpose scratch
-// of the fallback network), and a separate 4 KB output staging buffer (output
-// word p at word p; the rounds run buckets 32..63 first, so rows 0..31 are
-// still live while the first round stages its output).
+// Per warp: 64 bucket counters (256 B) and the slot buffer [64 buckets][36
+// words] of u32 keys (9 KB; slot p of bucket b at word 36 b + p: the 36-word
+// stride makes both the random single-word scatter and the 16-byte row gathers
+// of 8 consecutive lanes spread over all banks; also the 4 KB transpose
+// scratch of the fallback network). Output word p is staged at slot word
+// 1152 + p (rows 32..63): the first round sorts buckets 32..63, so those rows
+// are drained before any output is staged, and rows 0..31 stay intact for the
+// second round.
 constexpr int kBkCntBytes = 64 * 4;
 constexpr int kBkRowWords = 36;  // slot row of one bucket: 32 slots + 4 words of skew
 constexpr int kBkSlotBytes = 64 * kBkRowWords * 4;
-constexpr int kBkOutBytes = 1024 * 4;
-constexpr int kBkWarpBytes = kBkCntBytes + kBkSlotBytes + kBkOutBytes;
+constexpr int kBkStageWord = 32 * kBkRowWords;  // output word p at slot word kBkStageWord + p (n <= 1152)
+constexpr int kBkWarpBytes = kBkCntBytes + kBkSlotBytes;
 constexpr int kBkSmemBytes = (kBkBlock / 32) * kBkWarpBytes;
 
 __device__ __forceinline__ float fmin_nan(float a, float b) {
@@ -120,6 +128,19 @@ __device__ __forceinline__ void sort32_bk(uint32_t (&k)[32], uint32_t one) {
   constexpr OddEvenTable<32> T{};
 #pragma unroll
   for (int c = 0; c < OddEvenTable<32>::C; ++c) {
+    if ((c % GAS_BK_MIX_DEN) < GAS_BK_MIX_NUM) ce<true>(k[T.e[c].a], k[T.e[c].b], one);
+    else ce<false>(k[T.e[c].a], k[T.e[c].b], one);
+  }
+}
+
+// Batcher's odd-even merge sort of the first NK registers (NK = 24, 28, 32;
+// checked exhaustively with the 0-1 principle). When registers NK..31 hold
+// keys that follow every key in 0..NK-1, the first NK outputs are sorted.
+template <int NK>
+__device__ __forceinline__ void sortn_bk(uint32_t (&k)[32], uint32_t one) {
+  constexpr OddEvenTable<NK> T{};
+#pragma unroll
+  for (int c = 0; c < OddEvenTable<NK>::C; ++c) {
     if ((c % GAS_BK_MIX_DEN) < GAS_BK_MIX_NUM) ce<true>(k[T.e[c].a], k[T.e[c].b], one);
     else ce<false>(k[T.e[c].a], k[T.e[c].b], one);
   }
@@ -183,15 +204,17 @@ __device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
 //     NaN sends the array to the fallback network.
 //  2. bucket counter b starts at the shared address of slot 0 of bucket row b
 //     and each key adds 4 to it: the atomic's old value IS the key's slot
-//     address (bucket row b, rank = arrival order).
-//  3. one store of 16 pad bytes at the row's first chunk past its keys, then
-//     the scatter (one store per key).
+//     address (bucket row b, rank = arrival order), and the key is stored
+//     there at once. A bucket of more than 32 keys sends the array to the
+//     fallback; its overflowing stores stay inside this warp's slot buffer
+//     (addresses are clamped to its last word).
+//  3. pad keys after the last key of each row, up to the next 16-byte chunk.
 //  4. rounds: lane l sorts bucket l + 32 first, then bucket l. Only the
 //     ceil(size/4) chunks holding keys are gathered: the other registers hold
 //     pads (first round) or the sorted keys of bucket l + 32 (second round),
 //     which all follow every key of bucket l (the map is monotone), so the
 //     first size_b network outputs are bucket b sorted in both rounds.
-//     Outputs are staged at words base_b + i of the output buffer.
+//     Outputs are staged at slot words kBkStageWord + base_b + i.
 //  5. coalesced in-place store (key -> bits for non-raw arrays).
 __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     k_fixed_bucket1024(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
@@ -200,7 +223,8 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
   const uint32_t cnt_sa = wsa;                               // counter of bucket b at cnt_sa + b*4
   const uint32_t slot_sa = wsa + kBkCntBytes;                // slot (p, b) at slot_sa + (36 b + p)*4
-  const uint32_t out_sa = slot_sa + kBkSlotBytes;            // output word p at out_sa + p*4
+  const uint32_t stage_sa = slot_sa + kBkStageWord * 4;      // output word p at stage_sa + p*4
+  const uint32_t slot_last = slot_sa + kBkSlotBytes - 4;     // clamp of the scatter addresses
   uint32_t* const slot_ptr = reinterpret_cast<uint32_t*>(reinterpret_cast<unsigned char*>(bk_smem) +
                                                          warp * kBkWarpBytes + kBkCntBytes);
   const int nc = n >> 2;  // 16-byte chunks per array (> 128)
@@ -208,7 +232,6 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
   const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;  // counter address = bucket bits * 4 + cnt_b0
   const uint32_t row0 = slot_sa + lane * (kBkRowWords * 4);  // this lane's rows: buckets lane, lane + 32
   const uint32_t row1 = row0 + 32 * (kBkRowWords * 4);
-  const uint4 pad4 = make_uint4(kPadKey, kPadKey, kPadKey, kPadKey);
 
   for (int64_t a = (int64_t)blockIdx.x * (kBkBlock / 32) + warp; a < N; a += nwarps) {
     uint4* const dst = reinterpret_cast<uint4*>(d + a * (int64_t)n);
@@ -259,23 +282,40 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     }
     const float vmin = __uint_as_float(umin), vmax = __uint_as_float(umax);
     const float range = __fsub_rn(vmax, vmin);
-    const float s = __fdiv_rn(61.0f, range);
+    const float s = __fdiv_rn((float)GAS_BK_TOP, range);
     use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
     if (use_buckets) {
       sts32(cnt_sa + lane * 4, row0);
       sts32(cnt_sa + 128 + lane * 4, row1);
       __syncwarp();
-      // ---- rank: the atomic returns the key's slot address
-      uint32_t sa[32];
+      // ---- rank + scatter: the atomic returns the key's slot address
+      if (raw) {
 #pragma unroll
-      for (int r = 0; r < 32; ++r)
-        sa[r] = atoms_add4_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+        for (int r = 0; r < 32; ++r) {
+          const bool v = (r >> 2) < 4 || lane + 32 * (r >> 2) < nc;
+          const uint32_t sa = atoms_add4_if(v, bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+          sts32_if(v, min(sa, slot_last), k[r]);
+        }
+      } else {
+#pragma unroll
+        for (int r = 0; r < 32; ++r) {
+          const bool v = (r >> 2) < 4 || lane + 32 * (r >> 2) < nc;
+          const uint32_t sa = atoms_add4_if(v, bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+          sts32_if(v, min(sa, slot_last), key_from_bits(k[r]));
+        }
+      }
       __syncwarp();
       t0 = (lds32(cnt_sa + lane * 4) - row0) >> 2;
       t1 = (lds32(cnt_sa + 128 + lane * 4) - row1) >> 2;
       use_buckets = __all_sync(0xffffffffu, t0 <= 32u && t1 <= 32u);
       if (use_buckets) {
+        // pads after the last key of each row, up to its 16-byte chunk boundary
+#pragma unroll
+        for (int j = 0; j < 3; ++j) {
+          sts32_if(((t0 + j) & 3u) != 0u, row0 + (t0 + j) * 4, kPadKey);
+          sts32_if(((t1 + j) & 3u) != 0u, row1 + (t1 + j) * 4, kPadKey);
+        }
         // bucket bases: exclusive scan of the 64 bucket sizes (two 16-bit halves)
         uint32_t x = t0 | (t1 << 16);
 #pragma unroll
@@ -286,18 +326,6 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         const uint32_t total_lo = __shfl_sync(0xffffffffu, x & 0xFFFFu, 31);
         base0 = (x & 0xFFFFu) - t0;
         base1 = total_lo + (x >> 16) - t1;
-        // pads after the last key of each row (t <= 32: chunk 8 is the row's skew)
-        sts128(row0 + (t0 >> 2) * 16, pad4);
-        sts128(row1 + (t1 >> 2) * 16, pad4);
-        __syncwarp();
-        // ---- scatter
-        if (raw) {
-#pragma unroll
-          for (int r = 0; r < 32; ++r) sts32_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, sa[r], k[r]);
-        } else {
-#pragma unroll
-          for (int r = 0; r < 32; ++r) sts32_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, sa[r], key_from_bits(k[r]));
-        }
         __syncwarp();
       }
     }
@@ -309,14 +337,15 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       for (int rho = 0; rho < 2; ++rho) {
         const uint32_t tb = rho ? t0 : t1;
         const uint32_t row = rho ? row0 : row1;
-        const uint32_t ob = out_sa + (rho ? base0 : base1) * 4;
+        const uint32_t ob = stage_sa + (rho ? base0 : base1) * 4;
         if (rho == 0) {
 #pragma unroll
           for (int i = 0; i < 32; ++i) k[i] = kPadKey;
         }
 #pragma unroll
         for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
-        sort32_bk(k, one);
+        __syncwarp();  // rows 32..63 are drained before any output is staged over them
+        sortn_bk<32>(k, one);
 #pragma unroll
         for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
       }
@@ -325,18 +354,19 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 #pragma unroll
         for (int q = 0; q < 8; ++q) {
           const int c = lane + 32 * q;
-          stg_cs_if(q < 4 || c < nc, dst + c, lds128(out_sa + c * 16));
+          stg_cs_if(q < 4 || c < nc, dst + c, lds128(stage_sa + c * 16));
         }
       } else {
 #pragma unroll
         for (int q = 0; q < 8; ++q) {
           const int c = lane + 32 * q;
-          uint4 v = lds128(out_sa + c * 16);
+          uint4 v = lds128(stage_sa + c * 16);
           v.x = bits_from_key(v.x); v.y = bits_from_key(v.y); v.z = bits_from_key(v.z); v.w = bits_from_key(v.w);
           stg_cs_if(q < 4 || c < nc, dst + c, v);
         }
       }
     } else {
+      __syncwarp();  // the fallback's scratch overlaps the slot buffer
       bucket1024_fallback(k, dst, nc, lane, slot_ptr, one);
     }
     __syncwarp();
