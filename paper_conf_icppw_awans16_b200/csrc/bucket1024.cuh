@@ -386,9 +386,15 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 #pragma unroll
         for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
         __syncwarp();  // rows 32..63 are drained before any output is staged over them
+#ifndef GAS_ABL_NONET  // ablation builds (timing only, wrong output): skip the network / the staging
         sortn_bk<32>(k, one);
+#endif
+#ifndef GAS_ABL_NOSTAGE
 #pragma unroll
         for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
+#else
+        if (tb == 77) sts32(ob, k[0] + k[1] + k[5] + k[31]);
+#endif
       }
       __syncwarp();
       if (raw) {

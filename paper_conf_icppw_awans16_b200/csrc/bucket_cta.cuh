@@ -19,37 +19,55 @@
 
 namespace gas {
 
-template <int W>
+// One array per CTA of WR warps (T = 32 WR threads, 32 keys per thread,
+// n <= 1024 WR); W = the power of two >= WR whose whole-array network is the
+// fallback (sort_cta with W - WR virtual padding warps, warp1024.cuh).
+template <int W, int WR = W>
 struct BkCta {
-  static constexpr int T = 32 * W;         // threads
-  static constexpr int P = 1024 * W;       // capacity (keys)
-  static constexpr int NB = 62 * W;        // buckets 0 .. NB-1
-  static constexpr int ROWS = 64 * W;      // bucket rows (the last 2 W stay empty)
+  static_assert(WR <= W && 2 * WR > W, "W = the power of two covering WR");
+  static constexpr int T = 32 * WR;        // threads
+  static constexpr int P = 1024 * WR;      // capacity (keys)
+  static constexpr int ROWS = 64 * WR;     // bucket rows = buckets 0 .. ROWS-1
   static constexpr int CNT_BYTES = ROWS * 4;
   static constexpr int SLOT_BYTES = ROWS * kBkRowWords * 4;
-  static constexpr int RED_BYTES = 16 * 4;  // cross-warp min/max and scan partials
-  static constexpr int SMEM = CNT_BYTES + SLOT_BYTES + RED_BYTES;
-  // the fallback network needs P words of exchange + 4 KB per warp
-  static_assert(P * 4 + W * 4096 <= SLOT_BYTES, "fallback scratch fits in the slot buffer");
+  // the fallback network needs 1024 W words of exchange + 4 KB per warp
+  static constexpr int FB_BYTES = 1024 * W * 4 + WR * 4096;
+  static constexpr int BUF_BYTES = SLOT_BYTES > FB_BYTES ? SLOT_BYTES : FB_BYTES;
+  static constexpr int RED_BYTES = 48 * 4;  // cross-warp min/max [0, 2 WR) and scan partials [32, 32 + WR)
+  static constexpr int SMEM = CNT_BYTES + BUF_BYTES + RED_BYTES;
+  static_assert(WR <= 16, "cross-warp scratch");
 };
 
-#ifndef GAS_BKC_WARPS_PER_SM
-#define GAS_BKC_WARPS_PER_SM 16
+// Resident warps per SM (the register budget follows): measured best 16 for
+// WR = 2 and 20 for WR = 1, 4 (n = 2000: 5.00 vs 5.07 ms; n = 4000: 5.49 vs 5.31 ms).
+#ifdef GAS_BKC_WARPS_PER_SM
+template <int WR> constexpr int bkc_warps_per_sm() { return GAS_BKC_WARPS_PER_SM; }
+#else
+template <int WR> constexpr int bkc_warps_per_sm() { return WR == 2 ? 16 : (WR == 3 ? 18 : (WR >= 8 ? 16 : 20)); }
 #endif
+template <int WR> constexpr int bkc_min_blocks() { return bkc_warps_per_sm<WR>() / WR > 0 ? bkc_warps_per_sm<WR>() / WR : 1; }
 
 // Sort the n keys at `arr` (P/2 < n <= P; VEC: 16-byte-aligned, n % 4 == 0)
-// in place. All T threads of the CTA call it; `sm` is BkCta<W>::SMEM bytes.
-template <int W, bool VEC>
+// in place. All T threads of the CTA call it; `sm` is BkCta<W, WR>::SMEM bytes.
+// The steps are those of k_fixed_bucket1024 (bucket1024.cuh): counters start
+// at their rows' addresses so the atomic returns the slot address, fused
+// scatter, pads only after each row's last key, gathers of the occupied
+// chunks (upper buckets first, their sorted keys then pad the lower round),
+// output staged over the drained rows T .. 2T-1.
+template <int W, int WR, bool VEC>
 __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int n, unsigned char* sm, uint32_t one) {
-  using C = BkCta<W>;
+  using C = BkCta<W, WR>;
   constexpr int T = C::T;
   const int t = threadIdx.x, lane = t & 31, warp = t >> 5;
   const uint32_t cnt_sa = (uint32_t)__cvta_generic_to_shared(sm);
   const uint32_t slot_sa = cnt_sa + C::CNT_BYTES;
+  const uint32_t stage_sa = slot_sa + T * kBkRowWords * 4;  // output word p at stage_sa + 4p (rows T .. 2T-1)
+  const uint32_t slot_last = slot_sa + C::SLOT_BYTES - 4;
   unsigned char* const slot_ptr = sm + C::CNT_BYTES;
-  float* const red = reinterpret_cast<float*>(sm + C::CNT_BYTES + C::SLOT_BYTES);
+  uint32_t* const red = reinterpret_cast<uint32_t*>(sm + C::CNT_BYTES + C::BUF_BYTES);
   const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;
-  const uint32_t slot_c0 = slot_sa - (uint32_t)kBkRowWords * cnt_sa;
+  const uint32_t row0 = slot_sa + t * (kBkRowWords * 4);  // rows of buckets t and t + T
+  const uint32_t row1 = row0 + T * (kBkRowWords * 4);
   const int nc = n >> 2;
   // key r of this thread: VEC element 4 (t + T (r/4)) + r%4, else element t + T r
   auto valid = [&](int r) -> bool {
@@ -57,67 +75,87 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
     return r < 16 || t + T * r < n;
   };
 
-  // ---- stage in (raw bits); slots past the end stay out of every step
+  // ---- stage in (raw bits); slots past the end repeat k[0] (always valid)
   uint32_t k[32];
   if constexpr (VEC) {
     const uint4* src = reinterpret_cast<const uint4*>(arr);
 #pragma unroll
     for (int q = 0; q < 8; ++q) {
-      uint4 v = make_uint4(0, 0, 0, 0);
-      if (valid(4 * q)) v = ld_stream(src + t + T * q);
+      const uint4 v = q < 4 ? ld_stream(src + t + T * q) : ldg_cs_if(valid(4 * q), src + t + T * q);
       k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
     }
   } else {
 #pragma unroll
     for (int r = 0; r < 32; ++r) k[r] = valid(r) ? ld_stream(arr + t + T * r) : 0u;
   }
-  // ---- min / max over the valid keys (NaN-propagating), then across the CTA
-  float vmin = __uint_as_float(k[0]), vmax = vmin;
 #pragma unroll
-  for (int r = 1; r < 16; ++r) {
-    vmin = fmin_nan(vmin, __uint_as_float(k[r]));
-    vmax = fmax_nan(vmax, __uint_as_float(k[r]));
+  for (int r = 16; r < 32; ++r) k[r] = valid(r) ? k[r] : k[0];
+  // ---- min / max of the raw bits, then (if needed) of the keys, across the CTA
+  uint32_t umin = k[0], umax = k[0];
+#pragma unroll
+  for (int r = 1; r < 31; r += 2) {
+    umin = __vimin3_u32(umin, k[r], k[r + 1]);
+    umax = __vimax3_u32(umax, k[r], k[r + 1]);
   }
-#pragma unroll
-  for (int r = 16; r < 32; ++r)
-    if (valid(r)) {
-      vmin = fmin_nan(vmin, __uint_as_float(k[r]));
-      vmax = fmax_nan(vmax, __uint_as_float(k[r]));
-    }
-#pragma unroll
-  for (int m = 16; m >= 1; m >>= 1) {
-    vmin = fmin_nan(vmin, __shfl_xor_sync(0xffffffffu, vmin, m));
-    vmax = fmax_nan(vmax, __shfl_xor_sync(0xffffffffu, vmax, m));
-  }
-  if constexpr (W > 1) {
-    if (lane == 0) { red[2 * warp] = vmin; red[2 * warp + 1] = vmax; }
+  umin = __reduce_min_sync(0xffffffffu, min(umin, k[31]));
+  umax = __reduce_max_sync(0xffffffffu, max(umax, k[31]));
+  if constexpr (WR > 1) {
+    if (lane == 0) { red[2 * warp] = umin; red[2 * warp + 1] = umax; }
     __syncthreads();
 #pragma unroll
-    for (int w = 0; w < W; ++w) {
-      vmin = fmin_nan(vmin, red[2 * w]);
-      vmax = fmax_nan(vmax, red[2 * w + 1]);
-    }
+    for (int w = 0; w < WR; ++w) { umin = min(umin, red[2 * w]); umax = max(umax, red[2 * w + 1]); }
+    __syncthreads();
   }
+  const bool raw = umin > 0u && umax < 0x7F800000u;  // every value positive and finite (CTA-uniform)
+  bool use_buckets = true;
+  if (!raw) {
+    uint32_t kmin = 0xFFFFFFFFu, kmax = 0u;
+#pragma unroll
+    for (int r = 0; r < 32; ++r) {
+      const uint32_t kk = key_from_bits(k[r]);
+      kmin = min(kmin, kk);
+      kmax = max(kmax, kk);
+    }
+    kmin = __reduce_min_sync(0xffffffffu, kmin);
+    kmax = __reduce_max_sync(0xffffffffu, kmax);
+    if constexpr (WR > 1) {
+      if (lane == 0) { red[2 * warp] = kmin; red[2 * warp + 1] = kmax; }
+      __syncthreads();
+#pragma unroll
+      for (int w = 0; w < WR; ++w) { kmin = min(kmin, red[2 * w]); kmax = max(kmax, red[2 * w + 1]); }
+      __syncthreads();
+    }
+    use_buckets = kmin > 0x007FFFFFu && kmax < 0xFF800000u;  // no infinity, no NaN
+    umin = bits_from_key(kmin);
+    umax = bits_from_key(kmax);
+  }
+  const float vmin = __uint_as_float(umin), vmax = __uint_as_float(umax);
   const float range = __fsub_rn(vmax, vmin);
-  const float s = __fdiv_rn((float)(C::NB - 1), range);
-  bool use_buckets = fabsf(vmin) <= 3.402823466e38f && fabsf(vmax) <= 3.402823466e38f && range > 0.0f &&
-                     range <= 3.402823466e38f && s <= 3.402823466e38f;
-  const bool raw = vmin > 0.0f;
+  const float s = __fdiv_rn((float)(C::ROWS - 1), range);
+  use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
   uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
   if (use_buckets) {  // CTA-uniform
-#pragma unroll
-    for (int q = 0; q < C::SLOT_BYTES / 16 / T; ++q)
-      sts128(slot_sa + (t + T * q) * 16, make_uint4(kPadKey, kPadKey, kPadKey, kPadKey));
-    if (t < C::ROWS / 4) sts128(cnt_sa + t * 16, make_uint4(0, 0, 0, 0));
+    sts32(cnt_sa + t * 4, row0);
+    sts32(cnt_sa + (T + t) * 4, row1);
     __syncthreads();
-    uint32_t rk[32];
 #pragma unroll
-    for (int r = 0; r < 32; ++r) rk[r] = atoms_inc_if(valid(r), bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+    for (int g = 0; g < 32; g += 4) {
+      uint32_t sa[4];
+#pragma unroll
+      for (int r = g; r < g + 4; ++r) sa[r - g] = atoms_add4_if(valid(r), bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+#pragma unroll
+      for (int r = g; r < g + 4; ++r) sts32_if(valid(r), min(sa[r - g], slot_last), raw ? k[r] : key_from_bits(k[r]));
+    }
     __syncthreads();
-    t0 = lds32(cnt_sa + t * 4);
-    t1 = lds32(cnt_sa + (T + t) * 4);
+    t0 = (lds32(cnt_sa + t * 4) - row0) >> 2;
+    t1 = (lds32(cnt_sa + (T + t) * 4) - row1) >> 2;
     use_buckets = __syncthreads_and(t0 <= 32u && t1 <= 32u);
     if (use_buckets) {
+#pragma unroll
+      for (int j = 0; j < 3; ++j) {
+        sts32_if(((t0 + j) & 3u) != 0u, row0 + (t0 + j) * 4, kPadKey);
+        sts32_if(((t1 + j) & 3u) != 0u, row1 + (t1 + j) * 4, kPadKey);
+      }
       // bucket bases: exclusive scan of the 2T bucket sizes (two 16-bit halves)
       uint32_t x = t0 | (t1 << 16);
 #pragma unroll
@@ -126,13 +164,13 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
         if (lane >= m) x += y;
       }
       uint32_t before = 0, total = __shfl_sync(0xffffffffu, x, 31);
-      if constexpr (W > 1) {
-        uint32_t* const part = reinterpret_cast<uint32_t*>(red) + 8;
+      if constexpr (WR > 1) {
+        uint32_t* const part = red + 32;
         if (lane == 31) part[warp] = x;
         __syncthreads();
         total = 0;
 #pragma unroll
-        for (int w = 0; w < W; ++w) {
+        for (int w = 0; w < WR; ++w) {
           const uint32_t pw = part[w];
           before += (w < warp) ? pw : 0u;
           total += pw;
@@ -141,39 +179,27 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
       x += before;
       base0 = (x & 0xFFFFu) - t0;
       base1 = (total & 0xFFFFu) + (x >> 16) - t1;
-#pragma unroll
-      for (int r = 0; r < 32; ++r) {
-        const uint32_t ca = bucket_bits(k[r], vmin, s) * 4u + cnt_b0;
-        sts32_if(valid(r), ca * (uint32_t)kBkRowWords + (rk[r] * 4u + slot_c0), raw ? k[r] : key_from_bits(k[r]));
-      }
       __syncthreads();
     }
   }
 
   if (use_buckets) {
-    // two rounds: bucket t, then bucket t + T; the output is staged at word p
-    // of the slot buffer (rows 0 .. T-1 hold >= 36 T >= n words and are free
-    // after round 0's gather; round 1 reads rows T .. 2T-1 only)
-    const uint32_t out_sa = slot_sa;
+    // two rounds: bucket t + T, then bucket t
 #pragma unroll 1
     for (int rho = 0; rho < 2; ++rho) {
-      const uint32_t row = slot_sa + (t + T * rho) * (kBkRowWords * 4);
+      const uint32_t tb = rho ? t0 : t1;
+      const uint32_t row = rho ? row0 : row1;
+      const uint32_t ob = stage_sa + (rho ? base0 : base1) * 4;
+      if (rho == 0) {
 #pragma unroll
-      for (int q = 0; q < 8; ++q) {
-        const uint4 v = lds128(row + q * 16);
-        k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
+        for (int i = 0; i < 32; ++i) k[i] = kPadKey;
       }
-      __syncthreads();
-      sort32_bk(k, one);
-      const uint32_t tb = rho ? t1 : t0;
-      const uint32_t ob = out_sa + (rho ? base1 : base0) * 4;
-      if (raw) {
 #pragma unroll
-        for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
-      } else {
+      for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
+      __syncthreads();  // rows T .. 2T-1 are drained before any output is staged over them
+      sortn_bk<32>(k, one);
 #pragma unroll
-        for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, bits_from_key(k[i]));
-      }
+      for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
     }
     __syncthreads();
     if constexpr (VEC) {
@@ -181,13 +207,18 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
 #pragma unroll
       for (int q = 0; q < 8; ++q) {
         const int c = t + T * q;
-        if (c < nc) st_stream(dst + c, lds128(out_sa + c * 16));
+        uint4 v = lds128(stage_sa + c * 16);
+        if (!raw) { v.x = bits_from_key(v.x); v.y = bits_from_key(v.y); v.z = bits_from_key(v.z); v.w = bits_from_key(v.w); }
+        stg_cs_if(q < 4 || c < nc, dst + c, v);
       }
     } else {
 #pragma unroll
       for (int r = 0; r < 32; ++r) {
         const int e = t + T * r;
-        if (e < n) st_stream(arr + e, lds32(out_sa + e * 4));
+        if (e < n) {
+          const uint32_t v = lds32(stage_sa + e * 4);
+          st_stream(arr + e, raw ? v : bits_from_key(v));
+        }
       }
     }
   } else {
@@ -195,8 +226,9 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
 #pragma unroll
     for (int r = 0; r < 32; ++r) k[r] = valid(r) ? key_from_bits(k[r]) : kPadKey;
     uint32_t* xs = reinterpret_cast<uint32_t*>(slot_ptr);
-    uint32_t* wbuf = xs + C::P + warp * 1024;
+    uint32_t* wbuf = xs + 1024 * W + warp * 1024;
     __syncthreads();
+    fill_virtual<W, WR>(xs, t);
     sort_cta<W>(k, t, lane, xs, wbuf, one);
     __syncthreads();
     uint4* sb = reinterpret_cast<uint4*>(slot_ptr);
@@ -220,19 +252,19 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
 }
 
 // Fixed length, one array per CTA (persistent grid-stride).
-template <int W, bool VEC>
-__global__ void __launch_bounds__(32 * W, GAS_BKC_WARPS_PER_SM / W)
+template <int W, int WR, bool VEC>
+__global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
     k_fixed_bucket_cta(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   extern __shared__ __align__(16) unsigned char bkc_smem[];
-  for (int64_t a = blockIdx.x; a < N; a += gridDim.x) bucket_sort_cta<W, VEC>(d + a * (int64_t)n, n, bkc_smem, one);
+  for (int64_t a = blockIdx.x; a < N; a += gridDim.x) bucket_sort_cta<W, WR, VEC>(d + a * (int64_t)n, n, bkc_smem, one);
 }
 
 // Variable length: the arrays with LO < len <= HI (P/2 <= LO, HI <= P), found
 // by scanning windows of 32 arrays handed out dynamically through `ctr` (one
 // counter per launch, zeroed by the host), as k_offsets_cta. Rows may start
 // at any 4-byte boundary: scalar loads and stores.
-template <int W>
-__global__ void __launch_bounds__(32 * W, GAS_BKC_WARPS_PER_SM / W)
+template <int W, int WR>
+__global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
     k_offsets_bucket(uint32_t* __restrict__ d, const int64_t* __restrict__ off, int64_t N, int64_t LO, int64_t HI,
                      unsigned long long* __restrict__ ctr, uint32_t one) {
   extern __shared__ __align__(16) unsigned char bkc_smem[];
@@ -253,7 +285,7 @@ __global__ void __launch_bounds__(32 * W, GAS_BKC_WARPS_PER_SM / W)
       mask &= mask - 1;
       const int64_t lo = __shfl_sync(0xffffffffu, my_lo, pos);
       const int len = (int)__shfl_sync(0xffffffffu, my_len, pos);
-      bucket_sort_cta<W, false>(d + lo, len, bkc_smem, one);
+      bucket_sort_cta<W, WR, false>(d + lo, len, bkc_smem, one);
     }
   }
 }

@@ -86,24 +86,24 @@ bool bucket_enabled() {
 }
 
 // Bucket-then-network, one array per CTA of W warps (bucket_cta.cuh).
-template <int W, bool VEC>
+template <int W, int WR, bool VEC>
 cudaError_t launch_fixed_bucket_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  auto k = gas::k_fixed_bucket_cta<W, VEC>;
-  constexpr int smem = gas::BkCta<W>::SMEM;
+  auto k = gas::k_fixed_bucket_cta<W, WR, VEC>;
+  constexpr int smem = gas::BkCta<W, WR>::SMEM;
   const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
   if (e != cudaSuccess) return e;
-  k<<<persistent_grid_smem(k, 32 * W, smem, N), 32 * W, smem, s>>>(d, N, n, 1u);
+  k<<<persistent_grid_smem(k, 32 * WR, smem, N), 32 * WR, smem, s>>>(d, N, n, 1u);
   return cudaGetLastError();
 }
 
-template <int W>
+template <int W, int WR>
 cudaError_t launch_offsets_bucket(uint32_t* d, const int64_t* off, int64_t N, int64_t lo, int64_t hi,
                                   unsigned long long* ctr, cudaStream_t s) {
-  auto k = gas::k_offsets_bucket<W>;
-  constexpr int smem = gas::BkCta<W>::SMEM;
+  auto k = gas::k_offsets_bucket<W, WR>;
+  constexpr int smem = gas::BkCta<W, WR>::SMEM;
   const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
   if (e != cudaSuccess) return e;
-  k<<<persistent_grid_smem(k, 32 * W, smem, (N + 31) / 32), 32 * W, smem, s>>>(d, off, N, lo, hi, ctr, 1u);
+  k<<<persistent_grid_smem(k, 32 * WR, smem, (N + 31) / 32), 32 * WR, smem, s>>>(d, off, N, lo, hi, ctr, 1u);
   return cudaGetLastError();
 }
 
@@ -111,9 +111,14 @@ cudaError_t launch_offsets_bucket(uint32_t* d, const int64_t* off, int64_t N, in
 // warps rounded to the instantiated set (padding blocks are virtual, see sort_cta).
 template <bool VEC>
 cudaError_t dispatch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  if (bucket_enabled() && n <= 4096) {
-    if (n <= 2048) return launch_fixed_bucket_cta<2, VEC>(d, N, n, s);
-    return launch_fixed_bucket_cta<4, VEC>(d, N, n, s);
+  if (bucket_enabled()) {
+    if (n <= 2048) return launch_fixed_bucket_cta<2, 2, VEC>(d, N, n, s);
+    if (n <= 3072) return launch_fixed_bucket_cta<4, 3, VEC>(d, N, n, s);
+    if (n <= 4096) return launch_fixed_bucket_cta<4, 4, VEC>(d, N, n, s);
+    if (n <= 6144) return launch_fixed_bucket_cta<8, 6, VEC>(d, N, n, s);
+    if (n <= 8192) return launch_fixed_bucket_cta<8, 8, VEC>(d, N, n, s);
+    if (n <= 12288) return launch_fixed_bucket_cta<16, 12, VEC>(d, N, n, s);
+    return launch_fixed_bucket_cta<16, 16, VEC>(d, N, n, s);
   }
   if (n <= 2048) return launch_fixed_cta<2, 2, VEC>(d, N, n, s);
   if (n <= 3072) return launch_fixed_cta<4, 3, VEC>(d, N, n, s);
@@ -175,7 +180,7 @@ cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
       // the kernel is ALU/issue-bound, not latency-bound.
       if (VEC && env_flag("GAS_TMA")) return launch_fixed_1024_tma(d, N, n, s);
       if (VEC && bucket_enabled()) return launch_fixed_bucket1024(d, N, n, s);
-      if (!VEC && bucket_enabled() && n > 512) return launch_fixed_bucket_cta<1, false>(d, N, n, s);
+      if (!VEC && bucket_enabled() && n > 512) return launch_fixed_bucket_cta<1, 1, false>(d, N, n, s);
       return launch_fixed_warp<32, 32, VEC>(d, N, n, s);
     default: return dispatch_fixed_cta<VEC>(d, N, n, s);
   }
@@ -215,21 +220,29 @@ cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, i
     case 256: return launch_offsets_warp<32, 8>(d, off, N, s);
     case 512: return launch_offsets_warp<32, 16>(d, off, N, s);
     case 1024:
-      if (bucket_enabled()) return launch_offsets_bucket<1>(d, off, N, 512, 1024, ctr + 7, s);
+      if (bucket_enabled()) return launch_offsets_bucket<1, 1>(d, off, N, 512, 1024, ctr + 7, s);
       return launch_offsets_warp<32, 32>(d, off, N, s);
     case 2048:
-      if (bucket_enabled()) return launch_offsets_bucket<2>(d, off, N, 1024, 2048, ctr, s);
+      if (bucket_enabled()) return launch_offsets_bucket<2, 2>(d, off, N, 1024, 2048, ctr, s);
       return launch_offsets_cta<2, 2>(d, off, N, 1024, 2048, ctr, s);
     case 3072:
-      if (bucket_enabled()) return launch_offsets_bucket<4>(d, off, N, 2048, 3072, ctr + 1, s);
+      if (bucket_enabled()) return launch_offsets_bucket<4, 3>(d, off, N, 2048, 3072, ctr + 1, s);
       return launch_offsets_cta<4, 3>(d, off, N, 2048, 3072, ctr + 1, s);
     case 4096:
-      if (bucket_enabled()) return launch_offsets_bucket<4>(d, off, N, 3072, 4096, ctr + 2, s);
+      if (bucket_enabled()) return launch_offsets_bucket<4, 4>(d, off, N, 3072, 4096, ctr + 2, s);
       return launch_offsets_cta<4, 4>(d, off, N, 3072, 4096, ctr + 2, s);
-    case 6144: return launch_offsets_cta<8, 6>(d, off, N, 4096, 6144, ctr + 3, s);
-    case 8192: return launch_offsets_cta<8, 8>(d, off, N, 6144, 8192, ctr + 4, s);
-    case 12288: return launch_offsets_cta<16, 12>(d, off, N, 8192, 12288, ctr + 5, s);
-    case 16384: return launch_offsets_cta<16, 16>(d, off, N, 12288, 16384, ctr + 6, s);
+    case 6144:
+      if (bucket_enabled()) return launch_offsets_bucket<8, 6>(d, off, N, 4096, 6144, ctr + 3, s);
+      return launch_offsets_cta<8, 6>(d, off, N, 4096, 6144, ctr + 3, s);
+    case 8192:
+      if (bucket_enabled()) return launch_offsets_bucket<8, 8>(d, off, N, 6144, 8192, ctr + 4, s);
+      return launch_offsets_cta<8, 8>(d, off, N, 6144, 8192, ctr + 4, s);
+    case 12288:
+      if (bucket_enabled()) return launch_offsets_bucket<16, 12>(d, off, N, 8192, 12288, ctr + 5, s);
+      return launch_offsets_cta<16, 12>(d, off, N, 8192, 12288, ctr + 5, s);
+    case 16384:
+      if (bucket_enabled()) return launch_offsets_bucket<16, 16>(d, off, N, 12288, 16384, ctr + 6, s);
+      return launch_offsets_cta<16, 16>(d, off, N, 12288, 16384, ctr + 6, s);
   }
   return cudaErrorInvalidValue;
 }

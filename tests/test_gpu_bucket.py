@@ -28,15 +28,19 @@ def f32(a) -> np.ndarray:
     return np.asarray(a, dtype=np.float32).view(np.uint32)
 
 
-def spread_array(n: int, rng, heavy_bucket=None, heavy_count=0, heavy_values=None) -> np.ndarray:
-    """n values in [0, 61] with 0 and 61 present; optionally `heavy_count` keys
-    in bucket `heavy_bucket` (b = rint(v)); the rest spread over the other buckets."""
-    vals = [0.0, 61.0]
+TOP = 63  # the warp kernel's largest bucket index (GAS_BK_TOP, 64 buckets)
+
+
+def spread_array(n: int, rng, heavy_bucket=None, heavy_count=0, heavy_values=None, top=TOP) -> np.ndarray:
+    """n values in [0, top] with 0 and top present, so that the bucket map is
+    b = rint(v); optionally `heavy_count` keys in bucket `heavy_bucket`; the
+    rest spread over the other buckets."""
+    vals = [0.0, float(top)]
     if heavy_bucket is not None:
         hv = heavy_values if heavy_values is not None else np.full(heavy_count, float(heavy_bucket))
         vals += list(hv)
     rest = n - len(vals)
-    others = [b for b in range(1, 61) if b != heavy_bucket]
+    others = [b for b in range(1, top) if b != heavy_bucket]
     per = np.bincount(np.arange(rest) % len(others), minlength=len(others))
     assert per.max() <= 24
     for b, c in zip(others, per):
@@ -147,7 +151,7 @@ def test_bucket_sign_modes(lo, hi):
     np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
 
 
-# ---- CTA bucket kernels (bucket_cta.cuh): W = 1 (unaligned n <= 1024), 2, 4
+# ---- CTA bucket kernels (bucket_cta.cuh): WR = 1 (unaligned n <= 1024), 2, 3, 4, 6, 8, 12, 16 warps
 
 from tests.test_gpu_parity import gpu_sort_offsets  # noqa: E402
 
@@ -169,30 +173,34 @@ def test_bucket_cta_unaligned_warp_class(dist, n):
 
 
 @pytest.mark.parametrize("count", [32, 33])
-def test_bucket_cta_capacity_edge(count):
-    """n = 4000 (W = 4, 248 buckets): vmin = 0, vmax = 247 maps b(v) = rint(v)."""
-    rng = np.random.default_rng(100 + count)
-    rows = []
-    for i in range(16):
-        vals = [0.0, 247.0] + list(100.0 + rng.uniform(-0.49, 0.49, size=count))
-        rest = 4000 - len(vals)
-        others = [b for b in range(1, 247) if b != 100]
-        per = np.bincount(np.arange(rest) % len(others), minlength=len(others))
-        for b, c in zip(others, per):
-            vals += list(b + rng.uniform(-0.45, 0.45, size=c))
-        v = np.array(vals, dtype=np.float32)
-        rng.shuffle(v)
-        rows.append(v.view(np.uint32))
+@pytest.mark.parametrize("n,wr", [(4000, 4), (2500, 3), (7000, 8)])
+def test_bucket_cta_capacity_edge(count, n, wr):
+    """CTA of WR warps (64 WR buckets): vmin = 0, vmax = 64 WR - 1 maps b(v) = rint(v);
+    one bucket holds exactly `count` keys (32: bucket path, 33: fallback)."""
+    rng = np.random.default_rng(100 + count + n)
+    top = 64 * wr - 1
+    rows = [spread_array(n, rng, heavy_bucket=100, heavy_count=count,
+                         heavy_values=100.0 + rng.uniform(-0.49, 0.49, size=count), top=top) for _ in range(12)]
     host = np.stack(rows)
     np.testing.assert_array_equal(gpu_sort_fixed(host, lead=4), oracle_sorted(host))
 
 
+@pytest.mark.parametrize("n", [4097, 5000, 6144, 6145, 8000, 8192, 8193, 11000, 12288, 12289, 16000, 16384])
+@pytest.mark.parametrize("dist", ["paper_uniform", "special_mix", "dup16"])
+def test_bucket_cta_large(dist, n):
+    """CTA bucket classes WR = 6, 8, 12, 16 (fallback networks W = 8, 16)."""
+    host = datagen.fixed(dist, 7105, 0, 24, n)
+    expect = oracle_sorted(host)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=4), expect)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=1), expect)
+
+
 @pytest.mark.parametrize("dist", ["paper_uniform", "spectra_mz", "sorted", "special_mix", "spectra_intensity"])
 def test_bucket_offsets_classes(dist):
-    """Variable lengths through the 1024 / 2048 / 3072 / 4096 bucket classes,
-    every start alignment."""
+    """Variable lengths through the 1024 .. 16384 bucket classes, every start alignment."""
     lens = datagen.lengths(7103, 0, 2500, 400, 4096)
     lens[:6] = [513, 1024, 1025, 2048, 3073, 4096]
+    lens[6:14] = [4097, 6144, 6145, 8192, 8193, 12288, 12289, 16384]
     off = datagen.offsets_from_lengths(lens)
     data = datagen.ragged(dist, 7103, 0, off)
     expect = data.copy()
