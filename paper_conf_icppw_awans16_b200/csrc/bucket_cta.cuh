@@ -33,7 +33,8 @@ struct BkCta {
   // the fallback network needs 1024 W words of exchange + 4 KB per warp
   static constexpr int FB_BYTES = 1024 * W * 4 + WR * 4096;
   static constexpr int BUF_BYTES = SLOT_BYTES > FB_BYTES ? SLOT_BYTES : FB_BYTES;
-  static constexpr int RED_BYTES = 48 * 4;  // cross-warp min/max [0, 2 WR) and scan partials [32, 32 + WR)
+  // cross-warp scratch: raw-bit min/max [0, 2 WR), key min/max [32, 32 + 2 WR), scan partials [64, 64 + WR)
+  static constexpr int RED_BYTES = 96 * 4;
   static constexpr int SMEM = CNT_BYTES + BUF_BYTES + RED_BYTES;
   static_assert(WR <= 16, "cross-warp scratch");
 };
@@ -54,6 +55,12 @@ template <int WR> constexpr int bkc_min_blocks() { return bkc_warps_per_sm<WR>()
 // scatter, pads only after each row's last key, gathers of the occupied
 // chunks (upper buckets first, their sorted keys then pad the lower round),
 // output staged over the drained rows T .. 2T-1.
+template <int WR>
+__device__ __forceinline__ void bar_cta() {
+  if constexpr (WR > 1) __syncthreads();
+  else __syncwarp();
+}
+
 template <int W, int WR, bool VEC>
 __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int n, unsigned char* sm, uint32_t one) {
   using C = BkCta<W, WR>;
@@ -99,12 +106,18 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
   }
   umin = __reduce_min_sync(0xffffffffu, min(umin, k[31]));
   umax = __reduce_max_sync(0xffffffffu, max(umax, k[31]));
+  // Barriers: 5 or 6 per array. The previous array's last shared accesses (output
+  // staging reads) are ordered before this array's first row write by the
+  // barrier below; counters and `red` were last read several barriers ago.
+  sts32(cnt_sa + t * 4, row0);  // counter b starts at the address of row b
+  sts32(cnt_sa + (T + t) * 4, row1);
   if constexpr (WR > 1) {
     if (lane == 0) { red[2 * warp] = umin; red[2 * warp + 1] = umax; }
-    __syncthreads();
+  }
+  bar_cta<WR>();
+  if constexpr (WR > 1) {
 #pragma unroll
     for (int w = 0; w < WR; ++w) { umin = min(umin, red[2 * w]); umax = max(umax, red[2 * w + 1]); }
-    __syncthreads();
   }
   const bool raw = umin > 0u && umax < 0x7F800000u;  // every value positive and finite (CTA-uniform)
   bool use_buckets = true;
@@ -119,11 +132,10 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
     kmin = __reduce_min_sync(0xffffffffu, kmin);
     kmax = __reduce_max_sync(0xffffffffu, kmax);
     if constexpr (WR > 1) {
-      if (lane == 0) { red[2 * warp] = kmin; red[2 * warp + 1] = kmax; }
+      if (lane == 0) { red[32 + 2 * warp] = kmin; red[32 + 2 * warp + 1] = kmax; }
       __syncthreads();
 #pragma unroll
-      for (int w = 0; w < WR; ++w) { kmin = min(kmin, red[2 * w]); kmax = max(kmax, red[2 * w + 1]); }
-      __syncthreads();
+      for (int w = 0; w < WR; ++w) { kmin = min(kmin, red[32 + 2 * w]); kmax = max(kmax, red[32 + 2 * w + 1]); }
     }
     use_buckets = kmin > 0x007FFFFFu && kmax < 0xFF800000u;  // no infinity, no NaN
     umin = bits_from_key(kmin);
@@ -135,9 +147,6 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
   use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
   uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
   if (use_buckets) {  // CTA-uniform
-    sts32(cnt_sa + t * 4, row0);
-    sts32(cnt_sa + (T + t) * 4, row1);
-    __syncthreads();
 #pragma unroll
     for (int g = 0; g < 32; g += 4) {
       uint32_t sa[4];
@@ -146,7 +155,7 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
 #pragma unroll
       for (int r = g; r < g + 4; ++r) sts32_if(valid(r), min(sa[r - g], slot_last), raw ? k[r] : key_from_bits(k[r]));
     }
-    __syncthreads();
+    bar_cta<WR>();
     t0 = (lds32(cnt_sa + t * 4) - row0) >> 2;
     t1 = (lds32(cnt_sa + (T + t) * 4) - row1) >> 2;
     use_buckets = __syncthreads_and(t0 <= 32u && t1 <= 32u);
@@ -165,9 +174,9 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
       }
       uint32_t before = 0, total = __shfl_sync(0xffffffffu, x, 31);
       if constexpr (WR > 1) {
-        uint32_t* const part = red + 32;
+        uint32_t* const part = red + 64;
         if (lane == 31) part[warp] = x;
-        __syncthreads();
+        __syncthreads();  // also publishes the pads
         total = 0;
 #pragma unroll
         for (int w = 0; w < WR; ++w) {
@@ -176,10 +185,10 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
           total += pw;
         }
       }
+      else __syncwarp();  // publishes the pads
       x += before;
       base0 = (x & 0xFFFFu) - t0;
       base1 = (total & 0xFFFFu) + (x >> 16) - t1;
-      __syncthreads();
     }
   }
 
@@ -196,12 +205,14 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
       }
 #pragma unroll
       for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
-      __syncthreads();  // rows T .. 2T-1 are drained before any output is staged over them
+      // rows T .. 2T-1 are drained before any output is staged over them (the
+      // second round reads rows 0 .. T-1, which staging never touches)
+      if (rho == 0) bar_cta<WR>();
       sortn_bk<32>(k, one);
 #pragma unroll
       for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
     }
-    __syncthreads();
+    bar_cta<WR>();
     if constexpr (VEC) {
       uint4* dst = reinterpret_cast<uint4*>(arr);
 #pragma unroll
@@ -248,7 +259,8 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
       }
     }
   }
-  __syncthreads();  // the next array reuses the shared buffers
+  // no trailing barrier: the next array's first shared write to the rows
+  // follows its first barrier (see above)
 }
 
 // Fixed length, one array per CTA (persistent grid-stride).

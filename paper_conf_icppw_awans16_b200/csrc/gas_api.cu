@@ -43,12 +43,23 @@ int32_t size_class(int64_t n) {  // smallest power of two >= n, n >= 2
 
 // Persistent grid: enough blocks to cover the work, at most the number of
 // blocks that can be resident on all SMs at once (a multiple of the SM count).
+// GAS_GRID_CAP=k (testing knob): at most k blocks per persistent launch, so that
+// every block sorts many arrays back to back (tools/sanitize_cases.py).
+int64_t grid_cap() {
+  static const int64_t cap = [] {
+    const char* v = std::getenv("GAS_GRID_CAP");
+    return v ? (int64_t)std::atoll(v) : (int64_t)0;
+  }();
+  return cap;
+}
+
 template <typename K>
 int persistent_grid(K kernel, int threads, int64_t blocks_needed) {
   int per_sm = 0;
   if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kernel, threads, 0) != cudaSuccess || per_sm <= 0)
     per_sm = 1;
-  const int64_t cap = (int64_t)per_sm * num_sms();
+  int64_t cap = (int64_t)per_sm * num_sms();
+  if (grid_cap() > 0 && grid_cap() < cap) cap = grid_cap();
   return (int)(blocks_needed < cap ? (blocks_needed > 0 ? blocks_needed : 1) : cap);
 }
 
@@ -66,7 +77,8 @@ int persistent_grid_smem(K kernel, int threads, int smem, int64_t blocks_needed)
   int per_sm = 0;
   if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kernel, threads, smem) != cudaSuccess || per_sm <= 0)
     per_sm = 1;
-  const int64_t cap = (int64_t)per_sm * num_sms();
+  int64_t cap = (int64_t)per_sm * num_sms();
+  if (grid_cap() > 0 && grid_cap() < cap) cap = grid_cap();
   return (int)(blocks_needed < cap ? (blocks_needed > 0 ? blocks_needed : 1) : cap);
 }
 

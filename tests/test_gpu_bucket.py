@@ -220,3 +220,21 @@ def test_bucket_offsets_mixed_signs_and_network_agree(monkeypatch):
     np.testing.assert_array_equal(got, expect)
     monkeypatch.setenv("GAS_BUCKET", "0")
     np.testing.assert_array_equal(gpu_sort_offsets(data, off, lead=2), expect)
+
+
+@pytest.mark.parametrize("n,N,lead", [(700, 30000, 3), (2000, 12000, 4), (3000, 8000, 4), (5000, 4000, 1), (9000, 1500, 4)])
+def test_bucket_cta_many_arrays_per_cta(n, N, lead):
+    """N far above the persistent grid, so every CTA sorts many arrays back to back
+    (the kernels keep no trailing barrier between arrays)."""
+    host = datagen.fixed("paper_uniform", 7106, 0, N, n)
+    host[::7] = datagen.fixed("special_mix", 7107, 0, len(host[::7]), n)  # fallback arrays interleaved
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=lead), oracle_sorted(host))
+
+
+def test_bucket_offsets_many_arrays():
+    lens = datagen.lengths(7108, 0, 40000, 513, 4096)
+    off = datagen.offsets_from_lengths(lens)
+    data = datagen.ragged("paper_uniform", 7108, 0, off)
+    expect = data.copy()
+    oracle.sort_arrays_offsets_(expect, off)
+    np.testing.assert_array_equal(gpu_sort_offsets(data, off, lead=1), expect)
