@@ -88,6 +88,20 @@ def issue_roofline(kernel_hint: str, units_per_s: float, sm_mhz, n_sms: int):
             "warp_instr_per_array": per_unit, "source": "profiles/ncu_summary.json (ncu smsp__inst_executed.sum)"}
 
 
+def smem_roofline(kernel_hint: str, units_per_s: float, sm_mhz, n_sms: int):
+    """Shared-memory view of the same kernel (the bucket kernel's binding resource,
+    DESIGN.md §6): shared-memory wavefronts per array from the committed ncu capture
+    x arrays/s, against 1 wavefront (128 B)/clk/SM x SMs x the SM clock of the run."""
+    e = ncu_entry(kernel_hint)
+    if not e.get("smem_wavefronts_per_launch") or not sm_mhz:
+        return None
+    per_unit = e["smem_wavefronts_per_launch"] / e["arrays_per_launch"]
+    achieved = per_unit * units_per_s
+    peak = n_sms * sm_mhz * 1e6
+    return {"bound": "smem", "achieved": achieved, "peak": peak, "unit": "wavefronts/s", "frac": achieved / peak,
+            "wavefronts_per_array": per_unit, "source": "profiles/ncu_summary.json (ncu l1tex__data_pipe_lsu_wavefronts_mem_shared.sum)"}
+
+
 def ncu_traffic(kernel_hint: str):
     """Per-launch DRAM traffic of the dominant kernel from the committed ncu summary."""
     path = os.path.join(ROOT, "profiles", "ncu_summary.json")
@@ -423,6 +437,9 @@ def main():
             "issue_roofline": (issue_roofline(kernel_hint, value / world, clk.summary()["sm_mhz"],
                                               torch.cuda.get_device_properties(dev).multi_processor_count)
                                if not ragged and cfg["n"] == 1000 else None),
+            "smem_roofline": (smem_roofline(kernel_hint, value / world, clk.summary()["sm_mhz"],
+                                            torch.cuda.get_device_properties(dev).multi_processor_count)
+                              if not ragged and cfg["n"] == 1000 else None),
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches,
             "clocks": clk.summary(), "wall_ms_timed_loop": t_wall * 1e3, "per_step_ms": per_step,
             "self_check_sorted": ok,
