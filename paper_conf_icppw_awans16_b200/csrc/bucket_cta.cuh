@@ -55,6 +55,16 @@ template <int WR> constexpr int bkc_min_blocks() { return bkc_warps_per_sm<WR>()
 // scatter, pads only after each row's last key, gathers of the occupied
 // chunks (upper buckets first, their sorted keys then pad the lower round),
 // output staged over the drained rows T .. 2T-1.
+#ifndef GAS_BKC_PREFETCH
+#define GAS_BKC_PREFETCH 1
+#endif
+// One TMA bulk prefetch into L2 of the 16-byte-aligned cover of [p, p + words).
+__device__ __forceinline__ void prefetch_l2(const uint32_t* p, int64_t words) {
+  const uintptr_t a = reinterpret_cast<uintptr_t>(p) & ~(uintptr_t)15;
+  const uintptr_t e = (reinterpret_cast<uintptr_t>(p + words) + 15) & ~(uintptr_t)15;
+  asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a), "r"((uint32_t)(e - a)) : "memory");
+}
+
 template <int WR>
 __device__ __forceinline__ void bar_cta() {
   if constexpr (WR > 1) __syncthreads();
@@ -147,13 +157,24 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
   use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
   uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
   if (use_buckets) {  // CTA-uniform
+    if (raw) {
 #pragma unroll
-    for (int g = 0; g < 32; g += 4) {
-      uint32_t sa[4];
+      for (int g = 0; g < 32; g += 4) {
+        uint32_t sa[4];
 #pragma unroll
-      for (int r = g; r < g + 4; ++r) sa[r - g] = atoms_add4_if(valid(r), bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+        for (int r = g; r < g + 4; ++r) sa[r - g] = atoms_add4_if(valid(r), bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
 #pragma unroll
-      for (int r = g; r < g + 4; ++r) sts32_if(valid(r), min(sa[r - g], slot_last), raw ? k[r] : key_from_bits(k[r]));
+        for (int r = g; r < g + 4; ++r) sts32_if(valid(r), min(sa[r - g], slot_last), k[r]);
+      }
+    } else {
+#pragma unroll
+      for (int g = 0; g < 32; g += 4) {
+        uint32_t sa[4];
+#pragma unroll
+        for (int r = g; r < g + 4; ++r) sa[r - g] = atoms_add4_if(valid(r), bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+#pragma unroll
+        for (int r = g; r < g + 4; ++r) sts32_if(valid(r), min(sa[r - g], slot_last), key_from_bits(k[r]));
+      }
     }
     bar_cta<WR>();
     t0 = (lds32(cnt_sa + t * 4) - row0) >> 2;
@@ -223,12 +244,17 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
         stg_cs_if(q < 4 || c < nc, dst + c, v);
       }
     } else {
+      if (raw) {
 #pragma unroll
-      for (int r = 0; r < 32; ++r) {
-        const int e = t + T * r;
-        if (e < n) {
-          const uint32_t v = lds32(stage_sa + e * 4);
-          st_stream(arr + e, raw ? v : bits_from_key(v));
+        for (int r = 0; r < 32; ++r) {
+          const int e = t + T * r;
+          if (e < n) st_stream(arr + e, lds32(stage_sa + e * 4));
+        }
+      } else {
+#pragma unroll
+        for (int r = 0; r < 32; ++r) {
+          const int e = t + T * r;
+          if (e < n) st_stream(arr + e, bits_from_key(lds32(stage_sa + e * 4)));
         }
       }
     }
@@ -268,7 +294,12 @@ template <int W, int WR, bool VEC>
 __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
     k_fixed_bucket_cta(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   extern __shared__ __align__(16) unsigned char bkc_smem[];
-  for (int64_t a = blockIdx.x; a < N; a += gridDim.x) bucket_sort_cta<W, WR, VEC>(d + a * (int64_t)n, n, bkc_smem, one);
+  for (int64_t a = blockIdx.x; a < N; a += gridDim.x) {
+#if GAS_BKC_PREFETCH
+    if (threadIdx.x == 0 && a + gridDim.x < N) prefetch_l2(d + (a + gridDim.x) * (int64_t)n, n);
+#endif
+    bucket_sort_cta<W, WR, VEC>(d + a * (int64_t)n, n, bkc_smem, one);
+  }
 }
 
 // Variable length: the arrays with LO < len <= HI (P/2 <= LO, HI <= P), found
@@ -297,6 +328,14 @@ __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
       mask &= mask - 1;
       const int64_t lo = __shfl_sync(0xffffffffu, my_lo, pos);
       const int len = (int)__shfl_sync(0xffffffffu, my_len, pos);
+#if GAS_BKC_PREFETCH
+      if (mask) {  // warm L2 with the window's next array of this class
+        const int nx = __ffs(mask) - 1;
+        const int64_t nlo = __shfl_sync(0xffffffffu, my_lo, nx);
+        const int64_t nlen = __shfl_sync(0xffffffffu, my_len, nx);
+        if (t == 0) prefetch_l2(d + nlo, nlen);
+      }
+#endif
       bucket_sort_cta<W, WR, false>(d + lo, len, bkc_smem, one);
     }
   }
