@@ -328,6 +328,46 @@ struct HostStaging {
 };
 HostStaging g_staging[kMaxDevices];
 
+// Per-(device, caller stream) side streams of the offsets variant: the class
+// launches fork over them and join back (see gas_sort_arrays_offsets).
+constexpr int kMaxSide = 8;
+struct SideStreams {
+  cudaStream_t s[kMaxSide];
+  cudaEvent_t fork, join[kMaxSide];
+  std::mutex mu;
+};
+std::mutex g_side_mu;
+std::map<std::pair<int, cudaStream_t>, SideStreams*> g_side;
+
+int offsets_streams() {
+  static const int k = [] {
+    const char* v = std::getenv("GAS_OFFSETS_STREAMS");
+    const int x = v ? std::atoi(v) : 8;
+    return x < 1 ? 1 : (x > kMaxSide ? kMaxSide : x);
+  }();
+  return k;
+}
+
+cudaError_t side_streams_for(cudaStream_t stream, SideStreams** out) {
+  int dev = 0;
+  cudaError_t e = cudaGetDevice(&dev);
+  if (e != cudaSuccess) return e;
+  std::lock_guard<std::mutex> lock(g_side_mu);
+  auto& slot = g_side[{dev, stream}];
+  if (!slot) {
+    SideStreams* ss = new SideStreams();
+    e = cudaEventCreateWithFlags(&ss->fork, cudaEventDisableTiming);
+    for (int i = 0; i < kMaxSide && e == cudaSuccess; ++i) {
+      e = cudaStreamCreateWithFlags(&ss->s[i], cudaStreamNonBlocking);
+      if (e == cudaSuccess) e = cudaEventCreateWithFlags(&ss->join[i], cudaEventDisableTiming);
+    }
+    if (e != cudaSuccess) return e;  // (leaks the partial set; only on a failing device)
+    slot = ss;
+  }
+  *out = slot;
+  return cudaSuccess;
+}
+
 // Per-(device, stream) window counters of the offsets variant (see there).
 constexpr int kCounters = 8;
 std::mutex g_ctr_mu;
@@ -405,13 +445,41 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
   // size classes: 2, 4, ..., 2048 (len in (P/2, P]), then (2048, 3072] and (3072, 4096]
   const int32_t classes[] = {2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288, 16384};
   const int32_t lower[] = {1, 2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288};
-  for (int c = 0; c < 17; ++c) {
-    if (lower[c] >= max_array_len) break;
-    const cudaError_t e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, ctr, stream);
+  int nclass = 0;
+  while (nclass < 17 && lower[nclass] < max_array_len) ++nclass;
+  // The class launches are independent (disjoint arrays). With K > 1 they are
+  // forked over K streams (largest classes first) so that each persistent
+  // launch's last wave overlaps the next launches instead of idling SMs; the
+  // caller's stream waits for all of them (CUDA-graph capture follows the
+  // fork/join). GAS_OFFSETS_STREAMS=1 restores one stream.
+  SideStreams* ss = nullptr;
+  if (offsets_streams() > 1 && nclass > 1) {
+    const cudaError_t e = side_streams_for(stream, &ss);
     if (e != cudaSuccess) return cuda_fail(e);
-    g_launches.fetch_add(1, std::memory_order_relaxed);
   }
-  return GAS_SUCCESS;
+  if (!ss) {
+    for (int c = 0; c < nclass; ++c) {
+      const cudaError_t e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, ctr, stream);
+      if (e != cudaSuccess) return cuda_fail(e);
+      g_launches.fetch_add(1, std::memory_order_relaxed);
+    }
+    return GAS_SUCCESS;
+  }
+  std::lock_guard<std::mutex> lock(ss->mu);
+  const int K = offsets_streams();
+  cudaError_t e = cudaEventRecord(ss->fork, stream);
+  for (int i = 0; i < K && e == cudaSuccess; ++i) e = cudaStreamWaitEvent(ss->s[i], ss->fork, 0);
+  for (int c = nclass - 1, i = 0; c >= 0 && e == cudaSuccess; --c, ++i) {
+    e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, ctr, ss->s[i % K]);
+    if (e == cudaSuccess) g_launches.fetch_add(1, std::memory_order_relaxed);
+  }
+  // always join (also after an error) so that the caller's stream never races ahead
+  for (int i = 0; i < K; ++i) {
+    const cudaError_t r = cudaEventRecord(ss->join[i], ss->s[i]);
+    const cudaError_t w = r == cudaSuccess ? cudaStreamWaitEvent(stream, ss->join[i], 0) : r;
+    if (e == cudaSuccess) e = w;
+  }
+  return e == cudaSuccess ? GAS_SUCCESS : cuda_fail(e);
 }
 
 gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays, int32_t array_len,
