@@ -238,3 +238,53 @@ def test_bucket_offsets_many_arrays():
     expect = data.copy()
     oracle.sort_arrays_offsets_(expect, off)
     np.testing.assert_array_equal(gpu_sort_offsets(data, off, lead=1), expect)
+
+
+def _with_copies(n, rng, groups, top=TOP):
+    """spread_array-like rows where `groups` = [(value, count), ...] adds repeated keys."""
+    vals = [0.0, float(top)]
+    for v, c in groups:
+        vals += [v] * c
+    rest = n - len(vals)
+    heavy = {int(round(v)) for v, _ in groups}
+    others = [b for b in range(1, top) if b not in heavy]
+    per = np.bincount(np.arange(rest) % len(others), minlength=len(others))
+    for b, c in zip(others, per):
+        vals += list(b + rng.uniform(-0.45, 0.45, size=c))
+    v = np.array(vals, dtype=np.float32)
+    rng.shuffle(v)
+    return v.view(np.uint32)
+
+
+@pytest.mark.parametrize("case", ["one_key_33", "one_key_200", "two_one_key_buckets", "mixed_keys_fail",
+                                  "signed_one_key", "almost_all_equal"])
+def test_bucket_overflowing_repeated_keys(case):
+    """Buckets of more than 32 keys, one repeated key or several: the warp falls
+    back to the network, exactly (one-key retry measured slower and dropped)."""
+    rng = np.random.default_rng(sum(map(ord, case)))
+    rows = []
+    for i in range(48):
+        if case == "one_key_33":
+            r = _with_copies(1000, rng, [(17.0, 33)])
+        elif case == "one_key_200":
+            r = _with_copies(1000, rng, [(40.0, 200)])
+        elif case == "two_one_key_buckets":
+            r = _with_copies(1000, rng, [(5.0, 90), (50.0, 150)])
+        elif case == "mixed_keys_fail":  # two distinct keys in one overflowing bucket
+            r = _with_copies(1000, rng, [(30.0, 40), (30.25, 40)])
+        elif case == "signed_one_key":  # key path (negative values, a -0 / +0 bucket)
+            r = _with_copies(1000, rng, [(20.0, 100)])
+            r = (r.view(np.float32) - np.float32(31.0)).view(np.uint32)
+            r[:37] = np.float32(-0.0).view(np.uint32)
+        else:  # 998 copies of one value between the min and the max
+            r = np.full(1000, np.float32(5.0)).view(np.uint32)
+            r[rng.integers(0, 1000)] = np.float32(1.0).view(np.uint32)
+            r[rng.integers(0, 1000)] = np.float32(9.0).view(np.uint32)
+        rows.append(r)
+    host = np.stack(rows)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+def test_dup16_many_arrays():
+    host = datagen.fixed("dup16", 7109, 0, 20000, 1000)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
