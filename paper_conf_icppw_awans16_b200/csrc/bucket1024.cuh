@@ -63,6 +63,9 @@ namespace gas {
 #ifndef GAS_BK_INTERLEAVE  // 1: lane l sorts buckets 2l + 1, then 2l; 0: buckets l + 32, then l
 #define GAS_BK_INTERLEAVE 0
 #endif
+#ifndef GAS_BK_PREDICT  // 1 (skew) / 2 (skew + repeated samples): skip the bucket attempt when a 32-key sample predicts an overflow (off: see DESIGN.md §6)
+#define GAS_BK_PREDICT 0
+#endif
 #ifndef GAS_BK_PREFETCH
 #define GAS_BK_PREFETCH 1
 #endif
@@ -290,6 +293,31 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     const float range = __fsub_rn(vmax, vmin);
     const float s = __fdiv_rn((float)GAS_BK_TOP, range);
     use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
+#if GAS_BK_PREDICT
+    if (use_buckets) {
+      // Predicted overflow -> the network at once (saves the wasted bucket
+      // attempt on skewed or duplicate-heavy arrays). Sample: one key per
+      // lane from chunk lane % 8 (spread over the array); overflow is
+      // predicted when >= 12 of the 32 samples fall in the lowest or highest
+      // 8 of the 64 buckets (4 expected for a flat density), or one sample
+      // value occurs >= 3 times (essentially never for distinct values).
+      const int qs = lane & 7;
+      uint32_t x01 = (qs & 1) ? k[4] : k[0], x23 = (qs & 1) ? k[12] : k[8];
+      uint32_t x45 = (qs & 1) ? k[20] : k[16], x67 = (qs & 1) ? k[28] : k[24];
+      x01 = (qs & 2) ? x23 : x01;
+      x45 = (qs & 2) ? x67 : x45;
+      const uint32_t smp = (qs & 4) ? x45 : x01;
+      const float pos = __fmul_rn(__fsub_rn(__uint_as_float(smp), vmin), s);
+      const int lo = __popc(__ballot_sync(0xffffffffu, pos < 8.0f));
+      const int hi = __popc(__ballot_sync(0xffffffffu, pos > (float)(GAS_BK_TOP - 8)));
+#if GAS_BK_PREDICT > 1
+      const bool dup = __popc(__match_any_sync(0xffffffffu, smp)) >= 3;
+      use_buckets = lo < 12 && hi < 12 && !__any_sync(0xffffffffu, dup);
+#else
+      use_buckets = lo < 12 && hi < 12;
+#endif
+    }
+#endif
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
     if (use_buckets) {
 #if GAS_BK_INTERLEAVE
