@@ -40,10 +40,10 @@
 namespace gas {
 
 #ifndef GAS_BK_BLOCK
-#define GAS_BK_BLOCK 128
+#define GAS_BK_BLOCK 768  // one block of 24 warps per SM (80 registers): 4.22 ms; 20 warps as 640 / 320 / 160 / 128-thread blocks: 4.25 / 4.33 / 4.38 / 4.39 ms
 #endif
 #ifndef GAS_BK_WARPS_PER_SM
-#define GAS_BK_WARPS_PER_SM 20
+#define GAS_BK_WARPS_PER_SM 24
 #endif
 #ifndef GAS_BK_MIX_NUM  // compare-exchanges of the bucket networks in FMA form: NUM out of DEN
 #define GAS_BK_MIX_NUM 2
@@ -66,7 +66,7 @@ namespace gas {
 #ifndef GAS_BK_PREDICT  // 1 (skew) / 2 (skew + repeated samples): skip the bucket attempt when a 32-key sample predicts an overflow (off: see DESIGN.md §6)
 #define GAS_BK_PREDICT 0
 #endif
-#ifndef GAS_BK_PREFETCH
+#ifndef GAS_BK_PREFETCH  // L2 prefetch of the array this warp sorts GAS_BK_PREFETCH iterations ahead (0 = off)
 #define GAS_BK_PREFETCH 1
 #endif
 constexpr int kBkBlock = GAS_BK_BLOCK;
@@ -253,8 +253,8 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
     }
 #if GAS_BK_PREFETCH
-    if (lane == 0 && a + nwarps < N)  // warm L2 with this warp's next array (one TMA bulk prefetch)
-      asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + (a + nwarps) * (int64_t)n),
+    if (lane == 0 && a + GAS_BK_PREFETCH * nwarps < N)  // warm L2 with this warp's next array (one TMA bulk prefetch)
+      asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + (a + GAS_BK_PREFETCH * nwarps) * (int64_t)n),
                    "r"((uint32_t)n * 4u) : "memory");
 #endif
     // slots past the end repeat k[0] so that min / max need no predicates
