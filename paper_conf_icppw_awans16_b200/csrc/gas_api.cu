@@ -63,15 +63,6 @@ int persistent_grid(K kernel, int threads, int64_t blocks_needed) {
   return (int)(blocks_needed < cap ? (blocks_needed > 0 ? blocks_needed : 1) : cap);
 }
 
-template <int KPT, int G, bool VEC>
-cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  constexpr int arrays_per_block = (gas::kWarpBlock / 32) * (32 / G);
-  auto k = gas::k_fixed_warp<KPT, G, VEC>;
-  const int grid = persistent_grid(k, gas::kWarpBlock, (N + arrays_per_block - 1) / arrays_per_block);
-  k<<<grid, gas::kWarpBlock, 0, s>>>(d, N, n, 1u);
-  return cudaGetLastError();
-}
-
 template <typename K>
 int persistent_grid_smem(K kernel, int threads, int smem, int64_t blocks_needed) {
   int per_sm = 0;
@@ -81,6 +72,20 @@ int persistent_grid_smem(K kernel, int threads, int smem, int64_t blocks_needed)
   if (grid_cap() > 0 && grid_cap() < cap) cap = grid_cap();
   return (int)(blocks_needed < cap ? (blocks_needed > 0 ? blocks_needed : 1) : cap);
 }
+
+template <int KPT, int G, bool VEC>
+cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  constexpr int blk = gas::warp_block<G>();
+  constexpr int smem = gas::warp_smem_bytes<KPT, G>();
+  constexpr int arrays_per_block = (blk / 32) * (32 / G);
+  auto k = gas::k_fixed_warp<KPT, G, VEC>;
+  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  if (e != cudaSuccess) return e;
+  const int grid = persistent_grid_smem(k, blk, smem, (N + arrays_per_block - 1) / arrays_per_block);
+  k<<<grid, blk, smem, s>>>(d, N, n, 1u);
+  return cudaGetLastError();
+}
+
 
 template <int W, int WR, bool VEC>
 cudaError_t launch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
@@ -201,10 +206,14 @@ cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
 
 template <int KPT, int G>
 cudaError_t launch_offsets_warp(uint32_t* d, const int64_t* off, int64_t N, cudaStream_t s) {
+  constexpr int blk = gas::warp_block<G>();
+  constexpr int smem = gas::warp_smem_bytes<KPT, G>();
   auto k = gas::k_offsets_warp<KPT, G>;
+  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  if (e != cudaSuccess) return e;
   const int64_t windows = (N + 31) / 32;
-  const int grid = persistent_grid(k, gas::kWarpBlock, (windows + 7) / 8);
-  k<<<grid, gas::kWarpBlock, 0, s>>>(d, off, N, 1u);
+  const int grid = persistent_grid_smem(k, blk, smem, (windows + blk / 32 - 1) / (blk / 32));
+  k<<<grid, blk, smem, s>>>(d, off, N, 1u);
   return cudaGetLastError();
 }
 

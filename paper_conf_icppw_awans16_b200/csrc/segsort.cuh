@@ -43,7 +43,20 @@ constexpr int kWarpBlock = GAS_WARP_BLOCK;  // threads per block for the warp-le
 // on B200 (profiles/r01_variants_small_occupancy.txt): the 1024 class (G = 32)
 // and the 256 class (G = 8) run best at 2 blocks (<= 128 registers), the
 // others at 3 blocks (<= 85 registers, small spills).
-constexpr int warp_min_blocks(int G) { return (G == 32 || G == 8) ? GAS_WARP_MIN_BLOCKS : GAS_WARP_MIN_BLOCKS + 1; }
+__host__ __device__ constexpr int warp_min_blocks(int G) { return (G == 32 || G == 8) ? GAS_WARP_MIN_BLOCKS : GAS_WARP_MIN_BLOCKS + 1; }
+// GAS_WARP_BIG: the same warps per SM as one block (warp_min_blocks(G) x
+// kWarpBlock threads) instead of several kWarpBlock-thread blocks (the bucket
+// kernel measured 4.22 vs 4.39 ms for one 768-thread block per SM).
+#ifndef GAS_WARP_BIG
+#define GAS_WARP_BIG 1
+#endif
+// Measured (configs[1] shape, 1 B200): n=500 6.52 -> 6.16 ms, n=250 6.11 -> 5.89,
+// n=100 4.77 -> 4.53, but n=60 (G = 2) 3.34 -> 3.59: classes with G >= 4 only.
+template <int G> __host__ __device__ constexpr bool warp_big() { return GAS_WARP_BIG && G >= 4; }
+template <int G> __host__ __device__ constexpr int warp_block() { return warp_big<G>() ? warp_min_blocks(G) * kWarpBlock : kWarpBlock; }
+template <int G> __host__ __device__ constexpr int warp_block_min() { return warp_big<G>() ? 1 : warp_min_blocks(G); }
+template <int KPT> __host__ __device__ constexpr int warp_smem_chunks() { return 32 * KPT / 4 > 0 ? 32 * KPT / 4 : 1; }  // uint4 per warp
+template <int KPT, int G> __host__ __device__ constexpr int warp_smem_bytes() { return warp_block<G>() / 32 * warp_smem_chunks<KPT>() * 16; }
 
 // XOR swizzle of 16-byte chunks inside 128-byte rows: chunk c of a rank-order
 // buffer lives at physical chunk swz(c). Writes of 8 consecutive chunks per
@@ -117,16 +130,16 @@ __device__ __forceinline__ void stage_out_words(const uint32_t (&k)[KPT], uint4*
 
 // Warp-level classes: P = KPT * G <= 1024, GROUPS = 32 / G arrays per warp.
 template <int KPT, int G, bool VEC>
-__global__ void __launch_bounds__(kWarpBlock, warp_min_blocks(G)) k_fixed_warp(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+__global__ void __launch_bounds__(warp_block<G>(), warp_block_min<G>()) k_fixed_warp(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   constexpr int GROUPS = 32 / G;
   constexpr int P = KPT * G;
-  constexpr int WORDS = 32 * KPT;  // per warp
-  __shared__ uint4 smem[kWarpBlock / 32][WORDS / 4 > 0 ? WORDS / 4 : 1];
+  constexpr int BLK = warp_block<G>();
+  extern __shared__ uint4 warp_dsm[];  // warp_smem_bytes<KPT, G>()
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const int g = lane & (G - 1), grp = lane / G;
-  uint4* sb = smem[warp];
-  const int64_t nwarps = (int64_t)gridDim.x * (kWarpBlock / 32);
-  for (int64_t base = ((int64_t)blockIdx.x * (kWarpBlock / 32) + warp) * GROUPS; base < N; base += nwarps * GROUPS) {
+  uint4* sb = warp_dsm + warp * warp_smem_chunks<KPT>();
+  const int64_t nwarps = (int64_t)gridDim.x * (BLK / 32);
+  for (int64_t base = ((int64_t)blockIdx.x * (BLK / 32) + warp) * GROUPS; base < N; base += nwarps * GROUPS) {
     const int64_t a = base + grp;
     const bool valid = a < N;
     uint32_t k[KPT];
@@ -295,17 +308,17 @@ __device__ __forceinline__ bool in_class(int64_t len, int P) {
 }
 
 template <int KPT, int G>
-__global__ void __launch_bounds__(kWarpBlock, warp_min_blocks(G)) k_offsets_warp(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
+__global__ void __launch_bounds__(warp_block<G>(), warp_block_min<G>()) k_offsets_warp(uint32_t* __restrict__ d, const int64_t* __restrict__ off,
                                                           int64_t N, uint32_t one) {
   constexpr int GROUPS = 32 / G;
   constexpr int P = KPT * G;
-  constexpr int WORDS = 32 * KPT;
-  __shared__ uint4 smem[kWarpBlock / 32][WORDS / 4 > 0 ? WORDS / 4 : 1];
+  constexpr int BLK = warp_block<G>();
+  extern __shared__ uint4 warp_dsm[];  // warp_smem_bytes<KPT, G>()
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const int g = lane & (G - 1), grp = lane / G;
-  uint4* sb = smem[warp];
-  const int64_t nwarps = (int64_t)gridDim.x * (kWarpBlock / 32);
-  for (int64_t win = ((int64_t)blockIdx.x * (kWarpBlock / 32) + warp) * 32; win < N; win += nwarps * 32) {
+  uint4* sb = warp_dsm + warp * warp_smem_chunks<KPT>();
+  const int64_t nwarps = (int64_t)gridDim.x * (BLK / 32);
+  for (int64_t win = ((int64_t)blockIdx.x * (BLK / 32) + warp) * 32; win < N; win += nwarps * 32) {
     const int64_t mine = win + lane;
     int64_t my_lo = 0, my_len = 0;
     if (mine < N) { my_lo = off[mine]; my_len = off[mine + 1] - my_lo; }
