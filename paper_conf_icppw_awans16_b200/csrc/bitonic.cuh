@@ -25,6 +25,21 @@
 
 namespace gas {
 
+// Barrier of a thread group: bar == 0 -> the whole CTA (__syncthreads);
+// else named barrier (bar & 0xFF) over (bar >> 8) threads (several arrays
+// sorted by independent thread groups of one CTA, bucket_cta.cuh).
+__device__ __forceinline__ void group_sync(uint32_t bar) {
+  if (bar == 0) __syncthreads();
+  else asm volatile("bar.sync %0, %1;" ::"r"(bar & 0xFFu), "r"(bar >> 8) : "memory");
+}
+__device__ __forceinline__ bool group_and(bool v, uint32_t bar) {
+  if (bar == 0) return __syncthreads_and(v);
+  uint32_t r;
+  asm volatile("{\n\t.reg .pred p, q;\n\tsetp.ne.u32 p, %1, 0;\n\tbar.red.and.pred q, %2, %3, p;\n\tselp.u32 %0, 1, 0, q;\n\t}"
+               : "=r"(r) : "r"((uint32_t)v), "r"(bar & 0xFFu), "r"(bar >> 8) : "memory");
+  return r != 0;
+}
+
 template <int X>
 struct Log2 { static constexpr int value = 1 + Log2<X / 2>::value; };
 template <>
@@ -108,11 +123,11 @@ struct Bitonic {
   // Shared-memory exchange stage for partners in other warps. Element (t, r)
   // is stored at xs[r*T + t] (conflict-free for consecutive t).
   __device__ __forceinline__ static void smem_stage(T (&k)[KPT], T* xs, int t, int tmask,
-                                                    int rmask, bool upper) {
-    __syncthreads();
+                                                    int rmask, bool upper, uint32_t bar = 0) {
+    group_sync(bar);
 #pragma unroll
     for (int r = 0; r < KPT; ++r) xs[r * NT + t] = k[r];
-    __syncthreads();
+    group_sync(bar);
     // tmask >= 32: the partner is in another warp and `upper` is a warp bit, so
     // this branch is warp-uniform and each key costs one min or one max
     if (upper) {

@@ -42,11 +42,11 @@ struct BkCta {
 // Resident warps per SM (the register budget follows): measured best 16 for
 // WR = 2 and 20 for WR = 1, 4 (n = 2000: 5.00 vs 5.07 ms; n = 4000: 5.49 vs 5.31 ms).
 #ifdef GAS_BKC_WARPS_PER_SM
-template <int WR> constexpr int bkc_warps_per_sm() { return GAS_BKC_WARPS_PER_SM; }
+template <int WR> __host__ __device__ constexpr int bkc_warps_per_sm() { return GAS_BKC_WARPS_PER_SM; }
 #else
-template <int WR> constexpr int bkc_warps_per_sm() { return WR == 2 ? 16 : (WR == 3 ? 18 : (WR >= 8 ? 16 : 20)); }
+template <int WR> __host__ __device__ constexpr int bkc_warps_per_sm() { return WR == 2 ? 16 : (WR == 3 ? 18 : (WR >= 8 ? 16 : 20)); }
 #endif
-template <int WR> constexpr int bkc_min_blocks() { return bkc_warps_per_sm<WR>() / WR > 0 ? bkc_warps_per_sm<WR>() / WR : 1; }
+template <int WR> __host__ __device__ constexpr int bkc_min_blocks() { return bkc_warps_per_sm<WR>() / WR > 0 ? bkc_warps_per_sm<WR>() / WR : 1; }
 
 // Sort the n keys at `arr` (P/2 < n <= P; VEC: 16-byte-aligned, n % 4 == 0)
 // in place. All T threads of the CTA call it; `sm` is BkCta<W, WR>::SMEM bytes.
@@ -65,17 +65,35 @@ __device__ __forceinline__ void prefetch_l2(const uint32_t* p, int64_t words) {
   asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a), "r"((uint32_t)(e - a)) : "memory");
 }
 
+// Arrays per CTA: GROUPS independent thread groups of WR warps share one CTA
+// (one CTA per SM; GAS_BKC_GROUPS=0: one group per CTA, several CTAs per SM)
+// and synchronise with their own named barrier (group_sync, bitonic.cuh).
+#ifndef GAS_BKC_GROUPS
+#define GAS_BKC_GROUPS 1
+#endif
+// Measured (1 B200): grouped n=2500 5.76 -> 5.69 ms, 4000 5.07 -> 5.00, 8000
+// 6.39 -> 6.32, but n=2000 (WR = 2) 4.86 -> 5.14: groups for WR >= 3 only.
+template <int WR> __host__ __device__ constexpr bool bkc_grouped() { return GAS_BKC_GROUPS && WR >= 3; }
+template <int WR> __host__ __device__ constexpr int bkc_groups() { return bkc_grouped<WR>() ? bkc_min_blocks<WR>() : 1; }
+template <int WR> __host__ __device__ constexpr int bkc_block() { return 32 * WR * bkc_groups<WR>(); }
+template <int WR> __host__ __device__ constexpr int bkc_launch_min_blocks() { return bkc_grouped<WR>() ? 1 : bkc_min_blocks<WR>(); }
+static_assert(bkc_groups<2>() <= 15 && bkc_groups<3>() <= 15, "named barriers 1..15");
+
+// Barrier of the group (WR == 1: the warp).
 template <int WR>
-__device__ __forceinline__ void bar_cta() {
-  if constexpr (WR > 1) __syncthreads();
+__device__ __forceinline__ void bar_cta(uint32_t bar) {
+  if constexpr (WR > 1) group_sync(bar);
   else __syncwarp();
 }
 
+// t = thread index in the group (0 .. 32 WR - 1); bar = the group's barrier
+// (0: the group is the whole CTA).
 template <int W, int WR, bool VEC>
-__device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int n, unsigned char* sm, uint32_t one) {
+__device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int n, unsigned char* sm, uint32_t one,
+                                                int t, uint32_t bar) {
   using C = BkCta<W, WR>;
   constexpr int T = C::T;
-  const int t = threadIdx.x, lane = t & 31, warp = t >> 5;
+  const int lane = t & 31, warp = t >> 5;
   const uint32_t cnt_sa = (uint32_t)__cvta_generic_to_shared(sm);
   const uint32_t slot_sa = cnt_sa + C::CNT_BYTES;
   const uint32_t stage_sa = slot_sa + T * kBkRowWords * 4;  // output word p at stage_sa + 4p (rows T .. 2T-1)
@@ -124,7 +142,7 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
   if constexpr (WR > 1) {
     if (lane == 0) { red[2 * warp] = umin; red[2 * warp + 1] = umax; }
   }
-  bar_cta<WR>();
+  bar_cta<WR>(bar);
   if constexpr (WR > 1) {
 #pragma unroll
     for (int w = 0; w < WR; ++w) { umin = min(umin, red[2 * w]); umax = max(umax, red[2 * w + 1]); }
@@ -143,7 +161,7 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
     kmax = __reduce_max_sync(0xffffffffu, kmax);
     if constexpr (WR > 1) {
       if (lane == 0) { red[32 + 2 * warp] = kmin; red[32 + 2 * warp + 1] = kmax; }
-      __syncthreads();
+      group_sync(bar);
 #pragma unroll
       for (int w = 0; w < WR; ++w) { kmin = min(kmin, red[32 + 2 * w]); kmax = max(kmax, red[32 + 2 * w + 1]); }
     }
@@ -176,10 +194,11 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
         for (int r = g; r < g + 4; ++r) sts32_if(valid(r), min(sa[r - g], slot_last), key_from_bits(k[r]));
       }
     }
-    bar_cta<WR>();
+    bar_cta<WR>(bar);
     t0 = (lds32(cnt_sa + t * 4) - row0) >> 2;
     t1 = (lds32(cnt_sa + (T + t) * 4) - row1) >> 2;
-    use_buckets = __syncthreads_and(t0 <= 32u && t1 <= 32u);
+    if constexpr (WR > 1) use_buckets = group_and(t0 <= 32u && t1 <= 32u, bar);
+    else use_buckets = __all_sync(0xffffffffu, t0 <= 32u && t1 <= 32u);
     if (use_buckets) {
 #pragma unroll
       for (int j = 0; j < 3; ++j) {
@@ -197,7 +216,7 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
       if constexpr (WR > 1) {
         uint32_t* const part = red + 64;
         if (lane == 31) part[warp] = x;
-        __syncthreads();  // also publishes the pads
+        group_sync(bar);  // also publishes the pads
         total = 0;
 #pragma unroll
         for (int w = 0; w < WR; ++w) {
@@ -228,12 +247,12 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
       for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
       // rows T .. 2T-1 are drained before any output is staged over them (the
       // second round reads rows 0 .. T-1, which staging never touches)
-      if (rho == 0) bar_cta<WR>();
+      if (rho == 0) bar_cta<WR>(bar);
       sortn_bk<32>(k, one);
 #pragma unroll
       for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
     }
-    bar_cta<WR>();
+    bar_cta<WR>(bar);
     if constexpr (VEC) {
       uint4* dst = reinterpret_cast<uint4*>(arr);
 #pragma unroll
@@ -264,13 +283,13 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
     for (int r = 0; r < 32; ++r) k[r] = valid(r) ? key_from_bits(k[r]) : kPadKey;
     uint32_t* xs = reinterpret_cast<uint32_t*>(slot_ptr);
     uint32_t* wbuf = xs + 1024 * W + warp * 1024;
-    __syncthreads();
+    bar_cta<WR>(bar);
     fill_virtual<W, WR>(xs, t);
-    sort_cta<W>(k, t, lane, xs, wbuf, one);
-    __syncthreads();
+    sort_cta<W>(k, t, lane, xs, wbuf, one, bar);
+    bar_cta<WR>(bar);
     uint4* sb = reinterpret_cast<uint4*>(slot_ptr);
     stage_out_words<32>(k, sb, t * 32);
-    __syncthreads();
+    bar_cta<WR>(bar);
     if constexpr (VEC) {
 #pragma unroll
       for (int q = 0; q < 8; ++q) {
@@ -291,14 +310,19 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
 
 // Fixed length, one array per CTA (persistent grid-stride).
 template <int W, int WR, bool VEC>
-__global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
+__global__ void __launch_bounds__(bkc_block<WR>(), bkc_launch_min_blocks<WR>())
     k_fixed_bucket_cta(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   extern __shared__ __align__(16) unsigned char bkc_smem[];
-  for (int64_t a = blockIdx.x; a < N; a += gridDim.x) {
+  constexpr int GR = bkc_groups<WR>();
+  const int grp = threadIdx.x / (32 * WR), t = threadIdx.x % (32 * WR);
+  const uint32_t bar = GR > 1 ? (uint32_t)(grp + 1) | ((uint32_t)(32 * WR) << 8) : 0u;
+  unsigned char* const sm = bkc_smem + grp * BkCta<W, WR>::SMEM;
+  const int64_t stride = (int64_t)gridDim.x * GR;
+  for (int64_t a = (int64_t)blockIdx.x * GR + grp; a < N; a += stride) {
 #if GAS_BKC_PREFETCH
-    if (threadIdx.x == 0 && a + gridDim.x < N) prefetch_l2(d + (a + gridDim.x) * (int64_t)n, n);
+    if (t == 0 && a + stride < N) prefetch_l2(d + (a + stride) * (int64_t)n, n);
 #endif
-    bucket_sort_cta<W, WR, VEC>(d + a * (int64_t)n, n, bkc_smem, one);
+    bucket_sort_cta<W, WR, VEC>(d + a * (int64_t)n, n, sm, one, t, bar);
   }
 }
 
@@ -306,18 +330,24 @@ __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
 // by scanning windows of 32 arrays handed out dynamically through `ctr` (one
 // counter per launch, zeroed by the host), as k_offsets_cta. Rows may start
 // at any 4-byte boundary: scalar loads and stores.
+// (One group per CTA here: several small CTAs per SM co-reside with the other
+// size classes' launches on the forked streams; grouped CTAs measured slower on
+// configs[3], 6.13 vs 6.05 ms.)
 template <int W, int WR>
 __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
     k_offsets_bucket(uint32_t* __restrict__ d, const int64_t* __restrict__ off, int64_t N, int64_t LO, int64_t HI,
                      unsigned long long* __restrict__ ctr, uint32_t one) {
   extern __shared__ __align__(16) unsigned char bkc_smem[];
-  __shared__ int64_t s_win;
-  const int t = threadIdx.x, g = t & 31;
+  constexpr int GR = 1;
+  __shared__ int64_t s_win[GR];
+  const int grp = threadIdx.x / (32 * WR), t = threadIdx.x % (32 * WR), g = t & 31;
+  const uint32_t bar = GR > 1 ? (uint32_t)(grp + 1) | ((uint32_t)(32 * WR) << 8) : 0u;
+  unsigned char* const sm = bkc_smem + grp * BkCta<W, WR>::SMEM;
   for (;;) {
-    if (t == 0) s_win = (int64_t)atomicAdd(ctr, 1ull) * 32;
-    __syncthreads();
-    const int64_t win = s_win;
-    __syncthreads();
+    if (t == 0) s_win[grp] = (int64_t)atomicAdd(ctr, 1ull) * 32;
+    bar_cta<WR>(bar);
+    const int64_t win = s_win[grp];
+    bar_cta<WR>(bar);
     if (win >= N) break;
     const int64_t mine = win + g;
     int64_t my_lo = 0, my_len = 0;
@@ -336,7 +366,7 @@ __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
         if (t == 0) prefetch_l2(d + nlo, nlen);
       }
 #endif
-      bucket_sort_cta<W, WR, false>(d + lo, len, bkc_smem, one);
+      bucket_sort_cta<W, WR, false>(d + lo, len, sm, one, t, bar);
     }
   }
 }

@@ -106,10 +106,11 @@ bool bucket_enabled() {
 template <int W, int WR, bool VEC>
 cudaError_t launch_fixed_bucket_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   auto k = gas::k_fixed_bucket_cta<W, WR, VEC>;
-  constexpr int smem = gas::BkCta<W, WR>::SMEM;
+  constexpr int gr = gas::bkc_groups<WR>(), blk = gas::bkc_block<WR>();
+  constexpr int smem = gas::BkCta<W, WR>::SMEM * gr;
   const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
   if (e != cudaSuccess) return e;
-  k<<<persistent_grid_smem(k, 32 * WR, smem, N), 32 * WR, smem, s>>>(d, N, n, 1u);
+  k<<<persistent_grid_smem(k, blk, smem, (N + gr - 1) / gr), blk, smem, s>>>(d, N, n, 1u);
   return cudaGetLastError();
 }
 
@@ -117,10 +118,11 @@ template <int W, int WR>
 cudaError_t launch_offsets_bucket(uint32_t* d, const int64_t* off, int64_t N, int64_t lo, int64_t hi,
                                   unsigned long long* ctr, cudaStream_t s) {
   auto k = gas::k_offsets_bucket<W, WR>;
-  constexpr int smem = gas::BkCta<W, WR>::SMEM;
+  constexpr int gr = 1, blk = 32 * WR;
+  constexpr int smem = gas::BkCta<W, WR>::SMEM * gr;
   const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
   if (e != cudaSuccess) return e;
-  k<<<persistent_grid_smem(k, 32 * WR, smem, (N + 31) / 32), 32 * WR, smem, s>>>(d, off, N, lo, hi, ctr, 1u);
+  k<<<persistent_grid_smem(k, blk, smem, ((N + 31) / 32 + gr - 1) / gr), blk, smem, s>>>(d, off, N, lo, hi, ctr, 1u);
   return cudaGetLastError();
 }
 

@@ -181,14 +181,14 @@ __device__ __forceinline__ void cleaners1024_warp(uint32_t (&k)[32], int lane, u
 // network result for the real elements is unchanged.
 template <int W>
 __device__ __forceinline__ void sort_cta(uint32_t (&k)[32], int t, int lane, uint32_t* xs, uint32_t* wbuf,
-                                         uint32_t one) {
+                                         uint32_t one, uint32_t bar = 0) {
   using B = Bitonic<32, 32, W>;
   sort1024_warp(k, lane, wbuf, one);
 #pragma unroll 1
   for (int lk = 11; lk <= B::LOGP; ++lk) {
     const int K = 1 << lk;
-    B::smem_stage(k, xs, t, (K - 1) >> 5, 31, t & ((K >> 1) >> 5));  // mirror, across warps
-    for (int j = K >> 2; j >= 1024; j >>= 1) B::smem_stage(k, xs, t, j >> 5, 0, t & (j >> 5));
+    B::smem_stage(k, xs, t, (K - 1) >> 5, 31, t & ((K >> 1) >> 5), bar);  // mirror, across warps
+    for (int j = K >> 2; j >= 1024; j >>= 1) B::smem_stage(k, xs, t, j >> 5, 0, t & (j >> 5), bar);
     cleaners1024_warp(k, lane, wbuf, one);
   }
 }
