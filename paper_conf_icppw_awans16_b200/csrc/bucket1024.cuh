@@ -158,12 +158,14 @@ __device__ __forceinline__ void sortn_bk(uint32_t (&k)[32], uint32_t one) {
 // The whole-array network (warp1024.cuh) for arrays the bucket map cannot
 // handle. (Inline: an out-of-line call sends the key array through the stack
 // on every array, measured 84 local stores per array.)
+// QV: chunks q < QV are always inside the array (n > 128 QV).
+template <int QV = 4>
 __device__ __forceinline__ void bucket1024_fallback(uint32_t (&k)[32], uint4* dst, int nc, int lane, uint32_t* scratch,
                                                     uint32_t one) {
   __syncwarp();
 #pragma unroll
   for (int q = 0; q < 8; ++q) {
-    const bool valid = q < 4 || lane + 32 * q < nc;
+    const bool valid = q < QV || lane + 32 * q < nc;
 #pragma unroll
     for (int j = 0; j < 4; ++j) k[4 * q + j] = valid ? key_from_bits(k[4 * q + j]) : kPadKey;
   }

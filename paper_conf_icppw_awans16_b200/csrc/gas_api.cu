@@ -12,6 +12,7 @@
 #include "../../include/gas.h"
 #include "segsort.cuh"
 #include "bucket1024.cuh"
+#include "bucket512.cuh"
 #include "bucket_cta.cuh"
 #include "pairs.cuh"
 
@@ -181,6 +182,17 @@ cudaError_t launch_fixed_bucket1024(uint32_t* d, int64_t N, int n, cudaStream_t 
   return cudaGetLastError();
 }
 
+// Bucket-then-network kernel for 256 < n <= 512 with aligned rows (bucket512.cuh).
+cudaError_t launch_fixed_bucket512(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  const cudaError_t attr = cudaFuncSetAttribute(gas::k_fixed_bucket512, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                                gas::kBk5SmemBytes);
+  if (attr != cudaSuccess) return attr;
+  const int grid = persistent_grid_smem(gas::k_fixed_bucket512, gas::kBk5Block, gas::kBk5SmemBytes,
+                                        (N + GAS_BK5_WARPS - 1) / GAS_BK5_WARPS);
+  gas::k_fixed_bucket512<<<grid, gas::kBk5Block, gas::kBk5SmemBytes, s>>>(d, N, n, 1u);
+  return cudaGetLastError();
+}
+
 template <bool VEC>
 cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   switch (size_class(n)) {
@@ -192,7 +204,9 @@ cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
     case 64: return launch_fixed_warp<32, 2, VEC>(d, N, n, s);
     case 128: return launch_fixed_warp<32, 4, VEC>(d, N, n, s);
     case 256: return launch_fixed_warp<32, 8, VEC>(d, N, n, s);
-    case 512: return launch_fixed_warp<32, 16, VEC>(d, N, n, s);
+    case 512:
+      if (VEC && bucket_enabled()) return launch_fixed_bucket512(d, N, n, s);
+      return launch_fixed_warp<32, 16, VEC>(d, N, n, s);
     case 1024:
       // TMA-prefetch variant: opt-in (GAS_TMA=1). Measured on B200 it removes the
       // global-load stalls but is 5% slower overall (profiles/r01_ab_tma.txt):

@@ -288,3 +288,30 @@ def test_bucket_overflowing_repeated_keys(case):
 def test_dup16_many_arrays():
     host = datagen.fixed("dup16", 7109, 0, 20000, 1000)
     np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+# ---- bucket512.cuh: 256 < n <= 512 (16-byte rows), one warp per array, 32 buckets
+
+@pytest.mark.parametrize("n", [260, 300, 384, 500, 508, 512])
+@pytest.mark.parametrize("dist", ["paper_uniform", "spectra_mz", "sorted", "reverse", "spectra_intensity",
+                                  "dup16", "special_mix", "uniform_bits"])
+def test_bucket512_distributions(dist, n):
+    host = datagen.fixed(dist, 7110, 0, 700, n)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("count", [32, 33])
+def test_bucket512_capacity_edge(count):
+    rng = np.random.default_rng(300 + count)
+    rows = [spread_array(500, rng, heavy_bucket=9, heavy_count=count,
+                         heavy_values=9.0 + rng.uniform(-0.49, 0.49, size=count), top=31) for _ in range(64)]
+    host = np.stack(rows)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+def test_bucket512_many_arrays_and_unaligned():
+    host = datagen.fixed("paper_uniform", 7111, 0, 30000, 500)
+    host[::5] = datagen.fixed("dup16", 7112, 0, len(host[::5]), 500)  # fallback arrays interleaved
+    expect = oracle_sorted(host)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=4), expect)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=1), expect)  # network class (scalar path)
