@@ -181,6 +181,31 @@ __device__ __forceinline__ void bucket1024_fallback(uint32_t (&k)[32], uint4* ds
 }
 
 
+// any 4-byte alignment: key r of the lane is element lane + 32 r (n > 512)
+__device__ __forceinline__ void bucket1024_fallback_scalar(uint32_t (&k)[32], uint32_t* arr, int n, int lane,
+                                                           uint32_t* scratch, uint32_t one) {
+  __syncwarp();
+#pragma unroll
+  for (int r = 0; r < 32; ++r) k[r] = (r < 16 || lane + 32 * r < n) ? key_from_bits(k[r]) : kPadKey;
+  sort1024_warp(k, lane, scratch, one);
+  uint4* sb = reinterpret_cast<uint4*>(scratch);
+  stage_out<32>(k, sb, lane * 8);
+  __syncwarp();
+#pragma unroll
+  for (int r = 0; r < 32; ++r) {
+    const int e = lane + 32 * r;
+    if (e < n) st_stream(arr + e, sword(sb, e));
+  }
+}
+
+// One TMA bulk prefetch into L2 of the 16-byte-aligned cover of [p, p + words).
+__device__ __forceinline__ void prefetch_l2(const uint32_t* p, int64_t words) {
+  const uintptr_t a = reinterpret_cast<uintptr_t>(p) & ~(uintptr_t)15;
+  const uintptr_t e = (reinterpret_cast<uintptr_t>(p + words) + 15) & ~(uintptr_t)15;
+  asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a), "r"((uint32_t)(e - a)) : "memory");
+}
+
+
 // Predicated forms of the global / shared accesses of the kernel below (one
 // predicated instruction each instead of a branch around it).
 __device__ __forceinline__ uint4 ldg_cs_if(bool p, const uint4* a) {
@@ -445,6 +470,256 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     } else {
       __syncwarp();  // the fallback's scratch overlaps the slot buffer
       bucket1024_fallback(k, dst, nc, lane, slot_ptr, one);
+    }
+    __syncwarp();
+  }
+}
+
+// The same kernel for rows at any 4-byte alignment (n % 4 != 0 or an
+// unaligned base; instantiated with VEC = false): key r of a lane is element
+// lane + 32 r (4-byte accesses). Kept apart from k_fixed_bucket1024 so that the
+// 16-byte kernel's register allocation stays as measured (a merged template
+// spilled 12 bytes per array: 4.21 -> 4.31 ms).
+template <bool VEC>
+__global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
+    k_fixed_bucket1024_any(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+  extern __shared__ __align__(16) uint4 bk_smem[];
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
+  const uint32_t cnt_sa = wsa;                               // counter of bucket b at cnt_sa + b*4
+  const uint32_t slot_sa = wsa + kBkCntBytes;                // slot (p, b) at slot_sa + (36 b + p)*4
+  const uint32_t stage_sa = slot_sa + kBkStageWord * 4;      // output word p at stage_sa + p*4
+  const uint32_t slot_last = slot_sa + kBkSlotBytes - 4;     // clamp of the scatter addresses
+  uint32_t* const slot_ptr = reinterpret_cast<uint32_t*>(reinterpret_cast<unsigned char*>(bk_smem) +
+                                                         warp * kBkWarpBytes + kBkCntBytes);
+  const int nc = n >> 2;  // 16-byte chunks per array (> 128)
+  const int64_t nwarps = (int64_t)gridDim.x * (kBkBlock / 32);
+  const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;  // counter address = bucket bits * 4 + cnt_b0
+  const uint32_t row0 = slot_sa + lane * (kBkRowWords * 4);  // this lane's rows: buckets lane, lane + 32
+  const uint32_t row1 = row0 + 32 * (kBkRowWords * 4);
+
+  // key r of this lane lies inside the array (always for r < 16: n > 512)
+  auto valid = [&](int r) -> bool {
+    return VEC ? ((r >> 2) < 4 || lane + 32 * (r >> 2) < nc) : (r < 16 || lane + 32 * r < n);
+  };
+  for (int64_t a = (int64_t)blockIdx.x * (kBkBlock / 32) + warp; a < N; a += nwarps) {
+    uint32_t* const arr = d + a * (int64_t)n;
+    uint4* const dst = reinterpret_cast<uint4*>(arr);
+    // ---- a2: stage in (raw bits); keys r >= 16 may lie past the end (n > 512)
+    uint32_t k[32];
+    if constexpr (VEC) {
+#pragma unroll
+      for (int q = 0; q < 8; ++q) {
+        const int c = lane + 32 * q;
+        const uint4 v = q < 4 ? ld_stream(dst + c) : ldg_cs_if(c < nc, dst + c);
+        k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
+      }
+    } else {
+#pragma unroll
+      for (int r = 0; r < 32; ++r) k[r] = valid(r) ? ld_stream(arr + lane + 32 * r) : 0u;
+    }
+#if GAS_BK_PREFETCH
+    if (lane == 0 && a + GAS_BK_PREFETCH * nwarps < N) {  // warm L2 with this warp's next array (one TMA bulk prefetch)
+      if constexpr (VEC)
+        asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + (a + GAS_BK_PREFETCH * nwarps) * (int64_t)n),
+                     "r"((uint32_t)n * 4u) : "memory");
+      else
+        prefetch_l2(d + (a + GAS_BK_PREFETCH * nwarps) * (int64_t)n, n);
+    }
+#endif
+    // slots past the end repeat k[0] so that min / max need no predicates
+#pragma unroll
+    for (int r = 16; r < 32; ++r) k[r] = valid(r) ? k[r] : k[0];
+    // ---- bucket map parameters
+    uint32_t umin = k[0], umax = k[0];
+#pragma unroll
+    for (int r = 1; r < 31; r += 2) {
+      umin = __vimin3_u32(umin, k[r], k[r + 1]);
+      umax = __vimax3_u32(umax, k[r], k[r + 1]);
+    }
+    umin = __reduce_min_sync(0xffffffffu, min(umin, k[31]));
+    umax = __reduce_max_sync(0xffffffffu, max(umax, k[31]));
+    const bool raw = umin > 0u && umax < 0x7F800000u;  // every value positive and finite
+    bool use_buckets = true;
+    if (!raw) {  // min / max in key space; an infinity or NaN (either sign) -> fallback
+      uint32_t kmin = 0xFFFFFFFFu, kmax = 0u;
+#pragma unroll
+      for (int r = 0; r < 32; ++r) {
+        const uint32_t kk = key_from_bits(k[r]);
+        kmin = min(kmin, kk);
+        kmax = max(kmax, kk);
+      }
+      kmin = __reduce_min_sync(0xffffffffu, kmin);
+      kmax = __reduce_max_sync(0xffffffffu, kmax);
+      use_buckets = kmin > 0x007FFFFFu && kmax < 0xFF800000u;
+      umin = bits_from_key(kmin);
+      umax = bits_from_key(kmax);
+    }
+    const float vmin = __uint_as_float(umin), vmax = __uint_as_float(umax);
+    const float range = __fsub_rn(vmax, vmin);
+    const float s = __fdiv_rn((float)GAS_BK_TOP, range);
+    use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
+#if GAS_BK_PREDICT
+    if (use_buckets) {
+      // Predicted overflow -> the network at once (saves the wasted bucket
+      // attempt on skewed or duplicate-heavy arrays). Sample: one key per
+      // lane from chunk lane % 8 (spread over the array); overflow is
+      // predicted when >= 12 of the 32 samples fall in the lowest or highest
+      // 8 of the 64 buckets (4 expected for a flat density), or one sample
+      // value occurs >= 3 times (essentially never for distinct values).
+      const int qs = lane & 7;
+      uint32_t x01 = (qs & 1) ? k[4] : k[0], x23 = (qs & 1) ? k[12] : k[8];
+      uint32_t x45 = (qs & 1) ? k[20] : k[16], x67 = (qs & 1) ? k[28] : k[24];
+      x01 = (qs & 2) ? x23 : x01;
+      x45 = (qs & 2) ? x67 : x45;
+      const uint32_t smp = (qs & 4) ? x45 : x01;
+      const float pos = __fmul_rn(__fsub_rn(__uint_as_float(smp), vmin), s);
+      const int lo = __popc(__ballot_sync(0xffffffffu, pos < 8.0f));
+      const int hi = __popc(__ballot_sync(0xffffffffu, pos > (float)(GAS_BK_TOP - 8)));
+#if GAS_BK_PREDICT > 1
+      const bool dup = __popc(__match_any_sync(0xffffffffu, smp)) >= 3;
+      use_buckets = lo < 12 && hi < 12 && !__any_sync(0xffffffffu, dup);
+#else
+      use_buckets = lo < 12 && hi < 12;
+#endif
+    }
+#endif
+    uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
+    if (use_buckets) {
+#if GAS_BK_INTERLEAVE
+      // lane l owns buckets 2l (row l) and 2l + 1 (row 32 + l)
+      asm volatile("st.shared.v2.u32 [%0], {%1, %2};" ::"r"(cnt_sa + lane * 8), "r"(row0), "r"(row1) : "memory");
+#else
+      // lane l owns buckets l (row l) and l + 32 (row 32 + l)
+      sts32(cnt_sa + lane * 4, row0);
+      sts32(cnt_sa + 128 + lane * 4, row1);
+#endif
+      __syncwarp();
+      // ---- rank + scatter: the atomic returns the key's slot address
+      // (in groups of GAS_BK_GROUP keys: the atomics of a group are in flight together)
+      if (raw) {
+#pragma unroll
+        for (int g = 0; g < 32; g += GAS_BK_GROUP) {
+          uint32_t sa[GAS_BK_GROUP];
+#pragma unroll
+          for (int r = g; r < g + GAS_BK_GROUP; ++r)
+            sa[r - g] = atoms_add4_if(valid(r), bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+#pragma unroll
+          for (int r = g; r < g + GAS_BK_GROUP; ++r)
+            sts32_if(valid(r), min(sa[r - g], slot_last), k[r]);
+        }
+      } else {
+#pragma unroll
+        for (int g = 0; g < 32; g += GAS_BK_GROUP) {
+          uint32_t sa[GAS_BK_GROUP];
+#pragma unroll
+          for (int r = g; r < g + GAS_BK_GROUP; ++r)
+            sa[r - g] = atoms_add4_if(valid(r), bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+#pragma unroll
+          for (int r = g; r < g + GAS_BK_GROUP; ++r)
+            sts32_if(valid(r), min(sa[r - g], slot_last), key_from_bits(k[r]));
+        }
+      }
+      __syncwarp();
+#if GAS_BK_INTERLEAVE
+      {
+        uint32_t c0, c1;
+        asm volatile("ld.shared.v2.u32 {%0, %1}, [%2];" : "=r"(c0), "=r"(c1) : "r"(cnt_sa + lane * 8) : "memory");
+        t0 = (c0 - row0) >> 2;
+        t1 = (c1 - row1) >> 2;
+      }
+#else
+      t0 = (lds32(cnt_sa + lane * 4) - row0) >> 2;
+      t1 = (lds32(cnt_sa + 128 + lane * 4) - row1) >> 2;
+#endif
+      use_buckets = __all_sync(0xffffffffu, t0 <= 32u && t1 <= 32u);
+      if (use_buckets) {
+        // pads after the last key of each row, up to its 16-byte chunk boundary
+#pragma unroll
+        for (int j = 0; j < 3; ++j) {
+          sts32_if(((t0 + j) & 3u) != 0u, row0 + (t0 + j) * 4, kPadKey);
+          sts32_if(((t1 + j) & 3u) != 0u, row1 + (t1 + j) * 4, kPadKey);
+        }
+        // bucket bases: exclusive scan of the 64 bucket sizes (two 16-bit halves)
+#if GAS_BK_INTERLEAVE
+        uint32_t x = t0 + t1;  // inclusive scan of the lanes' bucket pairs
+#pragma unroll
+        for (int m = 1; m < 32; m <<= 1) {
+          const uint32_t y = __shfl_up_sync(0xffffffffu, x, m);
+          if (lane >= m) x += y;
+        }
+        base0 = x - t0 - t1;
+        base1 = base0 + t0;
+#else
+        uint32_t x = t0 | (t1 << 16);
+#pragma unroll
+        for (int m = 1; m < 32; m <<= 1) {
+          const uint32_t y = __shfl_up_sync(0xffffffffu, x, m);
+          if (lane >= m) x += y;
+        }
+        const uint32_t total_lo = __shfl_sync(0xffffffffu, x & 0xFFFFu, 31);
+        base0 = (x & 0xFFFFu) - t0;
+        base1 = total_lo + (x >> 16) - t1;
+#endif
+        __syncwarp();
+      }
+    }
+
+    if (use_buckets) {
+      // ---- two bucket rounds per lane (rolled: the hot code stays in the
+      // instruction cache): bucket lane + 32, then bucket lane
+#pragma unroll 1
+      for (int rho = 0; rho < 2; ++rho) {
+        const uint32_t tb = rho ? t0 : t1;
+        const uint32_t row = rho ? row0 : row1;
+        const uint32_t ob = stage_sa + (rho ? base0 : base1) * 4;
+        if (rho == 0) {
+#pragma unroll
+          for (int i = 0; i < 32; ++i) k[i] = kPadKey;
+        }
+#pragma unroll
+        for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
+        __syncwarp();  // rows 32..63 are drained before any output is staged over them
+#ifndef GAS_ABL_NONET  // ablation builds (timing only, wrong output): skip the network / the staging
+        sortn_bk<32>(k, one);
+#endif
+#ifndef GAS_ABL_NOSTAGE
+#pragma unroll
+        for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
+#else
+        if (tb == 77) sts32(ob, k[0] + k[1] + k[5] + k[31]);
+#endif
+      }
+      __syncwarp();
+      if constexpr (!VEC) {
+        if (raw) {
+#pragma unroll
+          for (int r = 0; r < 32; ++r)
+            if (valid(r)) st_stream(arr + lane + 32 * r, lds32(stage_sa + (lane + 32 * r) * 4));
+        } else {
+#pragma unroll
+          for (int r = 0; r < 32; ++r)
+            if (valid(r)) st_stream(arr + lane + 32 * r, bits_from_key(lds32(stage_sa + (lane + 32 * r) * 4)));
+        }
+      } else if (raw) {
+#pragma unroll
+        for (int q = 0; q < 8; ++q) {
+          const int c = lane + 32 * q;
+          stg_cs_if(q < 4 || c < nc, dst + c, lds128(stage_sa + c * 16));
+        }
+      } else {
+#pragma unroll
+        for (int q = 0; q < 8; ++q) {
+          const int c = lane + 32 * q;
+          uint4 v = lds128(stage_sa + c * 16);
+          v.x = bits_from_key(v.x); v.y = bits_from_key(v.y); v.z = bits_from_key(v.z); v.w = bits_from_key(v.w);
+          stg_cs_if(q < 4 || c < nc, dst + c, v);
+        }
+      }
+    } else {
+      __syncwarp();  // the fallback's scratch overlaps the slot buffer
+      if constexpr (VEC) bucket1024_fallback(k, dst, nc, lane, slot_ptr, one);
+      else bucket1024_fallback_scalar(k, arr, n, lane, slot_ptr, one);
     }
     __syncwarp();
   }

@@ -58,12 +58,6 @@ template <int WR> __host__ __device__ constexpr int bkc_min_blocks() { return bk
 #ifndef GAS_BKC_PREFETCH
 #define GAS_BKC_PREFETCH 1
 #endif
-// One TMA bulk prefetch into L2 of the 16-byte-aligned cover of [p, p + words).
-__device__ __forceinline__ void prefetch_l2(const uint32_t* p, int64_t words) {
-  const uintptr_t a = reinterpret_cast<uintptr_t>(p) & ~(uintptr_t)15;
-  const uintptr_t e = (reinterpret_cast<uintptr_t>(p + words) + 15) & ~(uintptr_t)15;
-  asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a), "r"((uint32_t)(e - a)) : "memory");
-}
 
 // Arrays per CTA: GROUPS independent thread groups of WR warps share one CTA
 // (one CTA per SM; GAS_BKC_GROUPS=0: one group per CTA, several CTAs per SM)

@@ -172,13 +172,14 @@ cudaError_t launch_fixed_1024_tma(uint32_t* d, int64_t N, int n, cudaStream_t s)
 
 // Bucket-then-network kernel for 512 < n <= 1024 with aligned rows
 // (bucket1024.cuh). Default on; GAS_BUCKET=0 selects the pure network.
+template <bool VEC>
 cudaError_t launch_fixed_bucket1024(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  const cudaError_t attr = cudaFuncSetAttribute(gas::k_fixed_bucket1024, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                                gas::kBkSmemBytes);
+  auto k = VEC ? gas::k_fixed_bucket1024 : gas::k_fixed_bucket1024_any<false>;
+  const cudaError_t attr = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kBkSmemBytes);
   if (attr != cudaSuccess) return attr;
-  const int grid = persistent_grid_smem(gas::k_fixed_bucket1024, gas::kBkBlock, gas::kBkSmemBytes,
+  const int grid = persistent_grid_smem(k, gas::kBkBlock, gas::kBkSmemBytes,
                                         (N + gas::kBkBlock / 32 - 1) / (gas::kBkBlock / 32));
-  gas::k_fixed_bucket1024<<<grid, gas::kBkBlock, gas::kBkSmemBytes, s>>>(d, N, n, 1u);
+  k<<<grid, gas::kBkBlock, gas::kBkSmemBytes, s>>>(d, N, n, 1u);
   return cudaGetLastError();
 }
 
@@ -212,8 +213,7 @@ cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
       // global-load stalls but is 5% slower overall (profiles/r01_ab_tma.txt):
       // the kernel is ALU/issue-bound, not latency-bound.
       if (VEC && env_flag("GAS_TMA")) return launch_fixed_1024_tma(d, N, n, s);
-      if (VEC && bucket_enabled()) return launch_fixed_bucket1024(d, N, n, s);
-      if (!VEC && bucket_enabled() && n > 512) return launch_fixed_bucket_cta<1, 1, false>(d, N, n, s);
+      if (bucket_enabled()) return launch_fixed_bucket1024<VEC>(d, N, n, s);
       return launch_fixed_warp<32, 32, VEC>(d, N, n, s);
     default: return dispatch_fixed_cta<VEC>(d, N, n, s);
   }

@@ -315,3 +315,13 @@ def test_bucket512_many_arrays_and_unaligned():
     expect = oracle_sorted(host)
     np.testing.assert_array_equal(gpu_sort_fixed(host, lead=4), expect)
     np.testing.assert_array_equal(gpu_sort_fixed(host, lead=1), expect)  # network class (scalar path)
+
+
+@pytest.mark.parametrize("n", [513, 515, 700, 999, 1021, 1023])
+@pytest.mark.parametrize("dist", ["paper_uniform", "special_mix", "dup16", "spectra_intensity"])
+def test_bucket_warp_unaligned(dist, n):
+    """k_fixed_bucket1024_any<false>: rows at any 4-byte alignment (n % 4 != 0 or an offset base)."""
+    host = datagen.fixed(dist, 7113, 0, 600, n)
+    expect = oracle_sorted(host)
+    for lead in (1, 2, 3):
+        np.testing.assert_array_equal(gpu_sort_fixed(host, lead=lead), expect)
