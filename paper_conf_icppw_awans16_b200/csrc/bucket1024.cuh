@@ -60,9 +60,6 @@ namespace gas {
 #ifndef GAS_BK_GROUP  // keys whose atomics are issued back to back before their scatter stores
 #define GAS_BK_GROUP 4
 #endif
-#ifndef GAS_BK_INTERLEAVE  // 1: lane l sorts buckets 2l + 1, then 2l; 0: buckets l + 32, then l
-#define GAS_BK_INTERLEAVE 0
-#endif
 #ifndef GAS_BK_PREDICT  // 1 (skew) / 2 (skew + repeated samples): skip the bucket attempt when a 32-key sample predicts an overflow (off: see DESIGN.md §6)
 #define GAS_BK_PREDICT 0
 #endif
@@ -347,14 +344,9 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 #endif
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
     if (use_buckets) {
-#if GAS_BK_INTERLEAVE
-      // lane l owns buckets 2l (row l) and 2l + 1 (row 32 + l)
-      asm volatile("st.shared.v2.u32 [%0], {%1, %2};" ::"r"(cnt_sa + lane * 8), "r"(row0), "r"(row1) : "memory");
-#else
       // lane l owns buckets l (row l) and l + 32 (row 32 + l)
       sts32(cnt_sa + lane * 4, row0);
       sts32(cnt_sa + 128 + lane * 4, row1);
-#endif
       __syncwarp();
       // ---- rank + scatter: the atomic returns the key's slot address
       // (in groups of GAS_BK_GROUP keys: the atomics of a group are in flight together)
@@ -382,17 +374,8 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         }
       }
       __syncwarp();
-#if GAS_BK_INTERLEAVE
-      {
-        uint32_t c0, c1;
-        asm volatile("ld.shared.v2.u32 {%0, %1}, [%2];" : "=r"(c0), "=r"(c1) : "r"(cnt_sa + lane * 8) : "memory");
-        t0 = (c0 - row0) >> 2;
-        t1 = (c1 - row1) >> 2;
-      }
-#else
       t0 = (lds32(cnt_sa + lane * 4) - row0) >> 2;
       t1 = (lds32(cnt_sa + 128 + lane * 4) - row1) >> 2;
-#endif
       use_buckets = __all_sync(0xffffffffu, t0 <= 32u && t1 <= 32u);
       if (use_buckets) {
         // pads after the last key of each row, up to its 16-byte chunk boundary
@@ -402,16 +385,6 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
           sts32_if(((t1 + j) & 3u) != 0u, row1 + (t1 + j) * 4, kPadKey);
         }
         // bucket bases: exclusive scan of the 64 bucket sizes (two 16-bit halves)
-#if GAS_BK_INTERLEAVE
-        uint32_t x = t0 + t1;  // inclusive scan of the lanes' bucket pairs
-#pragma unroll
-        for (int m = 1; m < 32; m <<= 1) {
-          const uint32_t y = __shfl_up_sync(0xffffffffu, x, m);
-          if (lane >= m) x += y;
-        }
-        base0 = x - t0 - t1;
-        base1 = base0 + t0;
-#else
         uint32_t x = t0 | (t1 << 16);
 #pragma unroll
         for (int m = 1; m < 32; m <<= 1) {
@@ -421,7 +394,6 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         const uint32_t total_lo = __shfl_sync(0xffffffffu, x & 0xFFFFu, 31);
         base0 = (x & 0xFFFFu) - t0;
         base1 = total_lo + (x >> 16) - t1;
-#endif
         __syncwarp();
       }
     }
@@ -586,14 +558,9 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 #endif
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
     if (use_buckets) {
-#if GAS_BK_INTERLEAVE
-      // lane l owns buckets 2l (row l) and 2l + 1 (row 32 + l)
-      asm volatile("st.shared.v2.u32 [%0], {%1, %2};" ::"r"(cnt_sa + lane * 8), "r"(row0), "r"(row1) : "memory");
-#else
       // lane l owns buckets l (row l) and l + 32 (row 32 + l)
       sts32(cnt_sa + lane * 4, row0);
       sts32(cnt_sa + 128 + lane * 4, row1);
-#endif
       __syncwarp();
       // ---- rank + scatter: the atomic returns the key's slot address
       // (in groups of GAS_BK_GROUP keys: the atomics of a group are in flight together)
@@ -621,17 +588,8 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         }
       }
       __syncwarp();
-#if GAS_BK_INTERLEAVE
-      {
-        uint32_t c0, c1;
-        asm volatile("ld.shared.v2.u32 {%0, %1}, [%2];" : "=r"(c0), "=r"(c1) : "r"(cnt_sa + lane * 8) : "memory");
-        t0 = (c0 - row0) >> 2;
-        t1 = (c1 - row1) >> 2;
-      }
-#else
       t0 = (lds32(cnt_sa + lane * 4) - row0) >> 2;
       t1 = (lds32(cnt_sa + 128 + lane * 4) - row1) >> 2;
-#endif
       use_buckets = __all_sync(0xffffffffu, t0 <= 32u && t1 <= 32u);
       if (use_buckets) {
         // pads after the last key of each row, up to its 16-byte chunk boundary
@@ -641,16 +599,6 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
           sts32_if(((t1 + j) & 3u) != 0u, row1 + (t1 + j) * 4, kPadKey);
         }
         // bucket bases: exclusive scan of the 64 bucket sizes (two 16-bit halves)
-#if GAS_BK_INTERLEAVE
-        uint32_t x = t0 + t1;  // inclusive scan of the lanes' bucket pairs
-#pragma unroll
-        for (int m = 1; m < 32; m <<= 1) {
-          const uint32_t y = __shfl_up_sync(0xffffffffu, x, m);
-          if (lane >= m) x += y;
-        }
-        base0 = x - t0 - t1;
-        base1 = base0 + t0;
-#else
         uint32_t x = t0 | (t1 << 16);
 #pragma unroll
         for (int m = 1; m < 32; m <<= 1) {
@@ -660,7 +608,6 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         const uint32_t total_lo = __shfl_sync(0xffffffffu, x & 0xFFFFu, 31);
         base0 = (x & 0xFFFFu) - t0;
         base1 = total_lo + (x >> 16) - t1;
-#endif
         __syncwarp();
       }
     }
