@@ -39,12 +39,19 @@ struct BkCta {
   static_assert(WR <= 16, "cross-warp scratch");
 };
 
-// Resident warps per SM (the register budget follows): measured best 16 for
-// WR = 2 and 20 for WR = 1, 4 (n = 2000: 5.00 vs 5.07 ms; n = 4000: 5.49 vs 5.31 ms).
+// Resident warps per SM (the register budget follows), measured: WR = 2: 18
+// (n = 2000: 4.69 ms vs 4.85 at 16, 4.77 at 20); WR = 3: 21 (n = 2500: 5.50 vs
+// 5.69 at 18); WR = 1, 4: 20 (SMEM caps WR = 4 at 20).
 #ifdef GAS_BKC_WARPS_PER_SM
 template <int WR> __host__ __device__ constexpr int bkc_warps_per_sm() { return GAS_BKC_WARPS_PER_SM; }
 #else
-template <int WR> __host__ __device__ constexpr int bkc_warps_per_sm() { return WR == 2 ? 16 : (WR == 3 ? 18 : (WR >= 8 ? 16 : 20)); }
+#ifndef GAS_BKC_W2
+#define GAS_BKC_W2 18
+#endif
+#ifndef GAS_BKC_W3
+#define GAS_BKC_W3 21
+#endif
+template <int WR> __host__ __device__ constexpr int bkc_warps_per_sm() { return WR == 2 ? GAS_BKC_W2 : (WR == 3 ? GAS_BKC_W3 : (WR >= 8 ? 16 : 20)); }
 #endif
 template <int WR> __host__ __device__ constexpr int bkc_min_blocks() { return bkc_warps_per_sm<WR>() / WR > 0 ? bkc_warps_per_sm<WR>() / WR : 1; }
 
