@@ -20,7 +20,7 @@
  * Conventions for every entry point:
  *   - Pointers named d_* are DEVICE memory of the current device, owned by
  *     the caller; gas_sort_arrays and gas_sort_pairs allocate nothing (zero
- *     workspace); the offsets variant keeps 64 bytes and 8 side streams per stream (see there); the library
+ *     workspace); the offsets variant keeps 72 bytes and 8 side streams per stream (see there); the library
  *     never calls cudaSetDevice.
  *   - Work is enqueued on `stream` (0 = legacy default stream) and the call
  *     returns without a host synchronisation. Argument and launch-
@@ -81,8 +81,8 @@ gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len,
  *                  on the device first (with a stream synchronisation) and a
  *                  violation returns GAS_ERROR_INVALID_VALUE with nothing sorted.
  *   max_array_len > gas_max_array_len(): GAS_ERROR_UNSUPPORTED.
- * Workspace: 64 bytes of device memory per (device, stream) for dynamic
- * scheduling when max_array_len > 512, allocated on the first such call and
+ * Workspace: 72 bytes of device memory per (device, stream) for dynamic
+ * scheduling when max_array_len > 256, allocated on the first such call and
  * kept (re-zeroed in stream order by every call).
  * One kernel launch per size class up to max_array_len (at most 17 launches:
  * powers of two up to 2048, then (2048,3072], (3072,4096], (4096,6144],

@@ -89,7 +89,9 @@ __device__ __forceinline__ void bar_cta(uint32_t bar) {
 
 // t = thread index in the group (0 .. 32 WR - 1); bar = the group's barrier
 // (0: the group is the whole CTA).
-template <int W, int WR, bool VEC>
+// RV: key slots r < RV are always inside the array (n > 32 WR RV; 16 for the
+// classes (P/2, P], 8 when the W = 1 kernel serves 256 < n <= 512).
+template <int W, int WR, bool VEC, int RV = 16>
 __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int n, unsigned char* sm, uint32_t one,
                                                 int t, uint32_t bar) {
   using C = BkCta<W, WR>;
@@ -108,7 +110,7 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
   // key r of this thread: VEC element 4 (t + T (r/4)) + r%4, else element t + T r
   auto valid = [&](int r) -> bool {
     if (VEC) return (r >> 2) < 4 || t + T * (r >> 2) < nc;
-    return r < 16 || t + T * r < n;
+    return r < RV || t + T * r < n;
   };
 
   // ---- stage in (raw bits); slots past the end repeat k[0] (always valid)
@@ -125,7 +127,7 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
     for (int r = 0; r < 32; ++r) k[r] = valid(r) ? ld_stream(arr + t + T * r) : 0u;
   }
 #pragma unroll
-  for (int r = 16; r < 32; ++r) k[r] = valid(r) ? k[r] : k[0];
+  for (int r = VEC ? 16 : RV; r < 32; ++r) k[r] = valid(r) ? k[r] : k[0];
   // ---- min / max of the raw bits, then (if needed) of the keys, across the CTA
   uint32_t umin = k[0], umax = k[0];
 #pragma unroll
@@ -334,7 +336,7 @@ __global__ void __launch_bounds__(bkc_block<WR>(), bkc_launch_min_blocks<WR>())
 // (One group per CTA here: several small CTAs per SM co-reside with the other
 // size classes' launches on the forked streams; grouped CTAs measured slower on
 // configs[3], 6.13 vs 6.05 ms.)
-template <int W, int WR>
+template <int W, int WR, int RV = 16>
 __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
     k_offsets_bucket(uint32_t* __restrict__ d, const int64_t* __restrict__ off, int64_t N, int64_t LO, int64_t HI,
                      unsigned long long* __restrict__ ctr, uint32_t one) {
@@ -367,7 +369,7 @@ __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
         if (t == 0) prefetch_l2(d + nlo, nlen);
       }
 #endif
-      bucket_sort_cta<W, WR, false>(d + lo, len, sm, one, t, bar);
+      bucket_sort_cta<W, WR, false, RV>(d + lo, len, sm, one, t, bar);
     }
   }
 }

@@ -98,6 +98,11 @@ cudaError_t launch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   return cudaGetLastError();
 }
 
+bool offsets512_bucket() {  // GAS_OFFSETS512=0: the (256, 512] offsets class on the network kernel
+  const char* v = std::getenv("GAS_OFFSETS512");
+  return !(v && std::strcmp(v, "0") == 0);
+}
+
 bool bucket_enabled() {
   const char* v = std::getenv("GAS_BUCKET");
   return !(v && std::strcmp(v, "0") == 0);
@@ -115,10 +120,10 @@ cudaError_t launch_fixed_bucket_cta(uint32_t* d, int64_t N, int n, cudaStream_t 
   return cudaGetLastError();
 }
 
-template <int W, int WR>
+template <int W, int WR, int RV = 16>
 cudaError_t launch_offsets_bucket(uint32_t* d, const int64_t* off, int64_t N, int64_t lo, int64_t hi,
                                   unsigned long long* ctr, cudaStream_t s) {
-  auto k = gas::k_offsets_bucket<W, WR>;
+  auto k = gas::k_offsets_bucket<W, WR, RV>;
   constexpr int gr = 1, blk = 32 * WR;
   constexpr int smem = gas::BkCta<W, WR>::SMEM * gr;
   const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
@@ -255,7 +260,9 @@ cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, i
     case 64: return launch_offsets_warp<32, 2>(d, off, N, s);
     case 128: return launch_offsets_warp<32, 4>(d, off, N, s);
     case 256: return launch_offsets_warp<32, 8>(d, off, N, s);
-    case 512: return launch_offsets_warp<32, 16>(d, off, N, s);
+    case 512:
+      if (bucket_enabled() && offsets512_bucket()) return launch_offsets_bucket<1, 1, 8>(d, off, N, 256, 512, ctr + 8, s);
+      return launch_offsets_warp<32, 16>(d, off, N, s);
     case 1024:
       if (bucket_enabled()) return launch_offsets_bucket<1, 1>(d, off, N, 512, 1024, ctr + 7, s);
       return launch_offsets_warp<32, 32>(d, off, N, s);
@@ -394,7 +401,7 @@ cudaError_t side_streams_for(cudaStream_t stream, SideStreams** out) {
 }
 
 // Per-(device, stream) window counters of the offsets variant (see there).
-constexpr int kCounters = 8;
+constexpr int kCounters = 9;
 std::mutex g_ctr_mu;
 std::map<std::pair<int, cudaStream_t>, unsigned long long*> g_ctr;
 
@@ -458,11 +465,11 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
     if (h) return GAS_ERROR_INVALID_VALUE;
   }
   uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
-  // 8 window counters for the CTA classes' dynamic scheduling: 64 bytes per
+  // 9 window counters for the bucket classes' dynamic scheduling: 72 bytes per
   // (device, stream), allocated on first use and re-zeroed in stream order by
   // every call (calls on one stream are ordered; different streams never share)
   unsigned long long* ctr = nullptr;
-  if (max_array_len > 512) {
+  if (max_array_len > 256) {
     cudaError_t e = counters_for(stream, &ctr);
     if (e == cudaSuccess) e = cudaMemsetAsync(ctr, 0, kCounters * sizeof(unsigned long long), stream);
     if (e != cudaSuccess) return cuda_fail(e);
