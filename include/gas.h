@@ -47,6 +47,15 @@
 extern "C" {
 #endif
 
+/* Exported symbols of libgas.so (built with -fvisibility=hidden: kernels and
+   helpers stay private, so a process can load several CUDA libraries that
+   share kernel names without interposition). */
+#if defined(__GNUC__)
+#define GAS_API __attribute__((visibility("default")))
+#else
+#define GAS_API
+#endif
+
 typedef enum gas_status {
   GAS_SUCCESS = 0,
   GAS_ERROR_INVALID_VALUE = 1, /* NULL pointer with work to do; negative count/length;
@@ -65,7 +74,7 @@ typedef enum gas_status {
  *   n > gas_max_array_len(): GAS_ERROR_UNSUPPORTED, nothing enqueued.
  * One kernel launch per call.
  */
-gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len, cudaStream_t stream);
+GAS_API gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len, cudaStream_t stream);
 
 /*
  * Variable-length batch (BASELINE.json north_star "variable-length offsets
@@ -93,7 +102,7 @@ gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len,
  * and the call can be captured into a CUDA graph. GAS_OFFSETS_STREAMS=k
  * (1..8) sets the fan-out; 1 keeps every launch on `stream`.
  */
-gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int64_t num_arrays,
+GAS_API gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int64_t num_arrays,
                                    int32_t max_array_len, cudaStream_t stream);
 
 /*
@@ -104,7 +113,7 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
  * gas_sort_arrays (both pointers 4-byte aligned), except that array_len is
  * limited to 8192 (GAS_ERROR_UNSUPPORTED above).
  */
-gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays, int32_t array_len,
+GAS_API gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays, int32_t array_len,
                           cudaStream_t stream);
 
 /*
@@ -120,21 +129,21 @@ gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays,
  * GAS_HOST_SLOTS) and its streams are allocated on first use per device and kept
  * for later calls; concurrent host-path calls on one device are serialised.
  */
-gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array_len);
+GAS_API gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array_len);
 
 /* Largest supported array length of gas_sort_arrays / _offsets / _host: 16384,
    4x the paper's spectra bound of ~4000 peaks. */
-int32_t gas_max_array_len(void);
+GAS_API int32_t gas_max_array_len(void);
 
 /* Static, human-readable name of a status code. */
-const char* gas_status_string(gas_status s);
+GAS_API const char* gas_status_string(gas_status s);
 
 /* cudaError_t of the most recent GAS_ERROR_CUDA on this host thread (0 if none). */
-int gas_last_cuda_error(void);
+GAS_API int gas_last_cuda_error(void);
 
 /* Number of kernels this library has launched in this process (monotone counter;
    bench.py reports the delta over its timed region as "gpu_launches"). */
-int64_t gas_launch_count(void);
+GAS_API int64_t gas_launch_count(void);
 
 #ifdef __cplusplus
 }

@@ -1,6 +1,12 @@
-"""Build libgas.so (the C-ABI library) in-tree for sm_100a with nvcc."""
+"""Build libgas.so (the C-ABI library) in-tree for sm_100a with nvcc.
+
+One translation unit per kernel family (csrc/k_*.cu) plus the API
+(csrc/gas_api.cu), compiled in parallel and linked into one shared library.
+Only the symbols of include/gas.h are exported (-fvisibility=hidden).
+"""
 from __future__ import annotations
 
+import concurrent.futures as cf
 import os
 import subprocess
 import sys
@@ -9,12 +15,13 @@ HERE = os.path.dirname(os.path.abspath(__file__))
 ROOT = os.path.dirname(HERE)
 CSRC = os.path.join(HERE, "csrc")
 OUT = os.path.join(HERE, "libgas.so")
-SOURCES = [os.path.join(CSRC, "gas_api.cu")]
+OBJ = os.path.join(ROOT, "build", "obj")
+SOURCES = [os.path.join(CSRC, f) for f in sorted(os.listdir(CSRC)) if f.endswith(".cu")]
 DEPS = SOURCES + [os.path.join(CSRC, f) for f in os.listdir(CSRC) if f.endswith((".cuh", ".h"))] + [
     os.path.join(ROOT, "include", "gas.h")]
 
 NVCC_FLAGS = ["-gencode", "arch=compute_100a,code=sm_100a", "-O3", "-lineinfo", "-std=c++17",
-              "-Xcompiler", "-fPIC", "-shared", "-Xptxas", "-warn-spills"]
+              "-Xcompiler", "-fPIC,-fvisibility=hidden", "-Xptxas", "-warn-spills"]
 
 
 def stale() -> bool:
@@ -24,15 +31,26 @@ def stale() -> bool:
     return any(os.path.getmtime(p) > t for p in DEPS)
 
 
-def build(force: bool = False, verbose: bool = False, extra=()) -> str:
-    if force or stale() or extra:
-        tmp = OUT + f".{os.getpid()}.tmp"
-        cmd = ["nvcc", *NVCC_FLAGS, *extra, "-I", os.path.join(ROOT, "include"), "-o", tmp, *SOURCES]
-        if verbose:
-            print(" ".join(cmd), file=sys.stderr)
-        subprocess.check_call(cmd)
-        os.replace(tmp, OUT)
-    return OUT
+def _compile(src: str, extra, verbose: bool) -> str:
+    obj = os.path.join(OBJ, os.path.basename(src)[:-3] + f".{os.getpid()}.o")
+    cmd = ["nvcc", *NVCC_FLAGS, *extra, "-I", os.path.join(ROOT, "include"), "-c", "-o", obj, src]
+    if verbose:
+        print(" ".join(cmd), file=sys.stderr)
+    subprocess.check_call(cmd)
+    return obj
+
+
+def build(force: bool = False, verbose: bool = False, extra=(), out: str = OUT) -> str:
+    if force or stale() or extra or out != OUT:
+        os.makedirs(OBJ, exist_ok=True)
+        with cf.ThreadPoolExecutor(max_workers=len(SOURCES)) as ex:
+            objs = list(ex.map(lambda s: _compile(s, extra, verbose), SOURCES))
+        tmp = out + f".{os.getpid()}.tmp"
+        subprocess.check_call(["nvcc", "-gencode", "arch=compute_100a,code=sm_100a", "-shared", "-o", tmp, *objs])
+        for o in objs:
+            os.remove(o)
+        os.replace(tmp, out)
+    return out
 
 
 if __name__ == "__main__":

@@ -60,9 +60,6 @@ namespace gas {
 #ifndef GAS_BK_GROUP  // keys whose atomics are issued back to back before their scatter stores
 #define GAS_BK_GROUP 4
 #endif
-#ifndef GAS_BK_PREDICT  // 1 (skew) / 2 (skew + repeated samples): skip the bucket attempt when a 32-key sample predicts an overflow (off: see DESIGN.md §6)
-#define GAS_BK_PREDICT 0
-#endif
 #ifndef GAS_BK_PREFETCH  // L2 prefetch of the array this warp sorts GAS_BK_PREFETCH iterations ahead (0 = off)
 #define GAS_BK_PREFETCH 1
 #endif
@@ -228,6 +225,60 @@ __device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
   return v;
 }
 
+// ---- Control block of the 512 < n <= 1024 pipeline (sort1024.cuh): device
+// workspace of one gas_sort_arrays call, followed by two array-index lists of
+// N entries each.
+enum : uint32_t { kS1Bucket = 0, kS1Count = 1, kS1Network = 2 };
+struct S1Ctl {
+  uint32_t votes[3];  // sampler: arrays voting for each path
+  uint32_t done;      // sampler blocks finished
+  uint32_t flag;      // the path that takes the whole batch (kS1*)
+  uint32_t n1;        // list 1: arrays the bucket kernel hands to the counting sort
+  uint32_t n2;        // list 2: arrays handed to the network
+  uint32_t pad;
+};
+__device__ __forceinline__ uint32_t* s1_list1(S1Ctl* c, int64_t N) { return reinterpret_cast<uint32_t*>(c + 1); }
+__device__ __forceinline__ uint32_t* s1_list2(S1Ctl* c, int64_t N) { return reinterpret_cast<uint32_t*>(c + 1) + N; }
+__device__ __forceinline__ void s1_push(uint32_t& count, uint32_t* list, int64_t a, int lane) {
+  if (lane == 0) list[atomicAdd(&count, 1u)] = (uint32_t)a;
+}
+
+#ifndef GAS_S1_PRED  // sample keys in one value bucket that send an array to the counting sort
+#define GAS_S1_PRED 5
+#endif
+// The 32-key sample of the predictors: one key per lane, spread over the
+// first 512 elements (which always exist, n > 512) so that pre-sorted arrays
+// do not look skewed: VEC layout, word 0 of chunk lane + 32 (lane & 3)
+// (element 4 lane + 128 (lane & 3)); scalar layout, element lane + 32 (lane & 15).
+template <bool VEC>
+__device__ __forceinline__ uint32_t bk_sample_key(const uint32_t (&k)[32], int lane) {
+  if constexpr (VEC) {
+    const uint32_t a = (lane & 1) ? k[4] : k[0], b = (lane & 1) ? k[12] : k[8];
+    return (lane & 2) ? b : a;
+  } else {
+    const uint32_t a0 = (lane & 1) ? k[1] : k[0], a1 = (lane & 1) ? k[3] : k[2];
+    const uint32_t a2 = (lane & 1) ? k[5] : k[4], a3 = (lane & 1) ? k[7] : k[6];
+    const uint32_t a4 = (lane & 1) ? k[9] : k[8], a5 = (lane & 1) ? k[11] : k[10];
+    const uint32_t a6 = (lane & 1) ? k[13] : k[12], a7 = (lane & 1) ? k[15] : k[14];
+    const uint32_t b0 = (lane & 2) ? a1 : a0, b1 = (lane & 2) ? a3 : a2;
+    const uint32_t b2 = (lane & 2) ? a5 : a4, b3 = (lane & 2) ? a7 : a6;
+    const uint32_t c0 = (lane & 4) ? b1 : b0, c1 = (lane & 4) ? b3 : b2;
+    return (lane & 8) ? c1 : c0;
+  }
+}
+
+// Overflow predictor of the value buckets: the 32-key sample k0 (one key per
+// lane) must not put >= 12 keys into the 8 lowest or the 8 highest buckets
+// (all-positive arrays: peaked values such as log-normal intensities), nor
+// >= GAS_S1_PRED keys into one bucket (other arrays: duplicates, zeros).
+__device__ __forceinline__ bool bk_sample_ok(uint32_t k0, bool raw, float vmin, float s) {
+  const uint32_t sb = bucket_bits(k0, vmin, s) - 0x4B000000u;
+  if (raw)
+    return __popc(__ballot_sync(0xffffffffu, sb < 8u)) < 12 &&
+           __popc(__ballot_sync(0xffffffffu, sb > (uint32_t)GAS_BK_TOP - 8u)) < 12;
+  return __reduce_max_sync(0xffffffffu, __popc(__match_any_sync(0xffffffffu, sb))) < GAS_S1_PRED;
+}
+
 // Fixed-length arrays, 512 < n <= 1024, 16-byte-aligned rows (n % 4 == 0).
 // One warp per array (persistent grid-stride). Per array:
 //  1. load (8 x LDG.128 per lane); min / max of the raw bits (VIMNMX3 + REDUX).
@@ -249,8 +300,8 @@ __device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
 //     first size_b network outputs are bucket b sorted in both rounds.
 //     Outputs are staged at slot words kBkStageWord + base_b + i.
 //  5. coalesced in-place store (key -> bits for non-raw arrays).
-__global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
-    k_fixed_bucket1024(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+static __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
+    k_fixed_bucket1024(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one, S1Ctl* ctl) {
   extern __shared__ __align__(16) uint4 bk_smem[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
@@ -265,6 +316,7 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
   const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;  // counter address = bucket bits * 4 + cnt_b0
   const uint32_t row0 = slot_sa + lane * (kBkRowWords * 4);  // this lane's rows: buckets lane, lane + 32
   const uint32_t row1 = row0 + 32 * (kBkRowWords * 4);
+  if (ctl && ctl->flag != kS1Bucket) return;  // pipeline: another kernel takes this batch
 
   for (int64_t a = (int64_t)blockIdx.x * (kBkBlock / 32) + warp; a < N; a += nwarps) {
     uint4* const dst = reinterpret_cast<uint4*>(d + a * (int64_t)n);
@@ -317,31 +369,9 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     const float range = __fsub_rn(vmax, vmin);
     const float s = __fdiv_rn((float)GAS_BK_TOP, range);
     use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
-#if GAS_BK_PREDICT
-    if (use_buckets) {
-      // Predicted overflow -> the network at once (saves the wasted bucket
-      // attempt on skewed or duplicate-heavy arrays). Sample: one key per
-      // lane from chunk lane % 8 (spread over the array); overflow is
-      // predicted when >= 12 of the 32 samples fall in the lowest or highest
-      // 8 of the 64 buckets (4 expected for a flat density), or one sample
-      // value occurs >= 3 times (essentially never for distinct values).
-      const int qs = lane & 7;
-      uint32_t x01 = (qs & 1) ? k[4] : k[0], x23 = (qs & 1) ? k[12] : k[8];
-      uint32_t x45 = (qs & 1) ? k[20] : k[16], x67 = (qs & 1) ? k[28] : k[24];
-      x01 = (qs & 2) ? x23 : x01;
-      x45 = (qs & 2) ? x67 : x45;
-      const uint32_t smp = (qs & 4) ? x45 : x01;
-      const float pos = __fmul_rn(__fsub_rn(__uint_as_float(smp), vmin), s);
-      const int lo = __popc(__ballot_sync(0xffffffffu, pos < 8.0f));
-      const int hi = __popc(__ballot_sync(0xffffffffu, pos > (float)(GAS_BK_TOP - 8)));
-#if GAS_BK_PREDICT > 1
-      const bool dup = __popc(__match_any_sync(0xffffffffu, smp)) >= 3;
-      use_buckets = lo < 12 && hi < 12 && !__any_sync(0xffffffffu, dup);
-#else
-      use_buckets = lo < 12 && hi < 12;
-#endif
-    }
-#endif
+    // pipeline mode (sort1024.cuh): arrays the 32-key sample predicts to
+    // overflow go to the counting sort without a bucket attempt
+    if (ctl && use_buckets) use_buckets = bk_sample_ok(bk_sample_key<true>(k, lane), raw, vmin, s);
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
     if (use_buckets) {
       // lane l owns buckets l (row l) and l + 32 (row 32 + l)
@@ -413,15 +443,9 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 #pragma unroll
         for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
         __syncwarp();  // rows 32..63 are drained before any output is staged over them
-#ifndef GAS_ABL_NONET  // ablation builds (timing only, wrong output): skip the network / the staging
         sortn_bk<32>(k, one);
-#endif
-#ifndef GAS_ABL_NOSTAGE
 #pragma unroll
         for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
-#else
-        if (tb == 77) sts32(ob, k[0] + k[1] + k[5] + k[31]);
-#endif
       }
       __syncwarp();
       if (raw) {
@@ -439,6 +463,8 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
           stg_cs_if(q < 4 || c < nc, dst + c, v);
         }
       }
+    } else if (ctl) {  // pipeline: the counting-sort kernel takes this array
+      s1_push(ctl->n1, s1_list1(ctl, N), a, lane);
     } else {
       __syncwarp();  // the fallback's scratch overlaps the slot buffer
       bucket1024_fallback(k, dst, nc, lane, slot_ptr, one);
@@ -454,7 +480,7 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 // spilled 12 bytes per array: 4.21 -> 4.31 ms).
 template <bool VEC>
 __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
-    k_fixed_bucket1024_any(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
+    k_fixed_bucket1024_any(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one, S1Ctl* ctl) {
   extern __shared__ __align__(16) uint4 bk_smem[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
@@ -469,6 +495,7 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
   const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;  // counter address = bucket bits * 4 + cnt_b0
   const uint32_t row0 = slot_sa + lane * (kBkRowWords * 4);  // this lane's rows: buckets lane, lane + 32
   const uint32_t row1 = row0 + 32 * (kBkRowWords * 4);
+  if (ctl && ctl->flag != kS1Bucket) return;  // pipeline: another kernel takes this batch
 
   // key r of this lane lies inside the array (always for r < 16: n > 512)
   auto valid = [&](int r) -> bool {
@@ -531,31 +558,9 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     const float range = __fsub_rn(vmax, vmin);
     const float s = __fdiv_rn((float)GAS_BK_TOP, range);
     use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
-#if GAS_BK_PREDICT
-    if (use_buckets) {
-      // Predicted overflow -> the network at once (saves the wasted bucket
-      // attempt on skewed or duplicate-heavy arrays). Sample: one key per
-      // lane from chunk lane % 8 (spread over the array); overflow is
-      // predicted when >= 12 of the 32 samples fall in the lowest or highest
-      // 8 of the 64 buckets (4 expected for a flat density), or one sample
-      // value occurs >= 3 times (essentially never for distinct values).
-      const int qs = lane & 7;
-      uint32_t x01 = (qs & 1) ? k[4] : k[0], x23 = (qs & 1) ? k[12] : k[8];
-      uint32_t x45 = (qs & 1) ? k[20] : k[16], x67 = (qs & 1) ? k[28] : k[24];
-      x01 = (qs & 2) ? x23 : x01;
-      x45 = (qs & 2) ? x67 : x45;
-      const uint32_t smp = (qs & 4) ? x45 : x01;
-      const float pos = __fmul_rn(__fsub_rn(__uint_as_float(smp), vmin), s);
-      const int lo = __popc(__ballot_sync(0xffffffffu, pos < 8.0f));
-      const int hi = __popc(__ballot_sync(0xffffffffu, pos > (float)(GAS_BK_TOP - 8)));
-#if GAS_BK_PREDICT > 1
-      const bool dup = __popc(__match_any_sync(0xffffffffu, smp)) >= 3;
-      use_buckets = lo < 12 && hi < 12 && !__any_sync(0xffffffffu, dup);
-#else
-      use_buckets = lo < 12 && hi < 12;
-#endif
-    }
-#endif
+    // pipeline mode (sort1024.cuh): arrays the 32-key sample predicts to
+    // overflow go to the counting sort without a bucket attempt
+    if (ctl && use_buckets) use_buckets = bk_sample_ok(bk_sample_key<VEC>(k, lane), raw, vmin, s);
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
     if (use_buckets) {
       // lane l owns buckets l (row l) and l + 32 (row 32 + l)
@@ -627,15 +632,9 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 #pragma unroll
         for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
         __syncwarp();  // rows 32..63 are drained before any output is staged over them
-#ifndef GAS_ABL_NONET  // ablation builds (timing only, wrong output): skip the network / the staging
         sortn_bk<32>(k, one);
-#endif
-#ifndef GAS_ABL_NOSTAGE
 #pragma unroll
         for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
-#else
-        if (tb == 77) sts32(ob, k[0] + k[1] + k[5] + k[31]);
-#endif
       }
       __syncwarp();
       if constexpr (!VEC) {
@@ -663,6 +662,8 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
           stg_cs_if(q < 4 || c < nc, dst + c, v);
         }
       }
+    } else if (ctl) {  // pipeline: the counting-sort kernel takes this array
+      s1_push(ctl->n1, s1_list1(ctl, N), a, lane);
     } else {
       __syncwarp();  // the fallback's scratch overlaps the slot buffer
       if constexpr (VEC) bucket1024_fallback(k, dst, nc, lane, slot_ptr, one);

@@ -24,7 +24,7 @@ constexpr int kBk5SlotBytes = 32 * kBkRowWords * 4;  // also the fallback networ
 constexpr int kBk5WarpBytes = kBk5CntBytes + kBk5SlotBytes;
 constexpr int kBk5SmemBytes = GAS_BK5_WARPS * kBk5WarpBytes;
 
-__global__ void __launch_bounds__(kBk5Block, 1)
+static __global__ void __launch_bounds__(kBk5Block, 1)
     k_fixed_bucket512(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   extern __shared__ __align__(16) uint4 bk5_smem[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;

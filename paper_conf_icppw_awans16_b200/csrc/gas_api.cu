@@ -10,11 +10,7 @@
 #include <cuda_runtime.h>
 
 #include "../../include/gas.h"
-#include "segsort.cuh"
-#include "bucket1024.cuh"
-#include "bucket512.cuh"
-#include "bucket_cta.cuh"
-#include "pairs.cuh"
+#include "launch_util.cuh"
 
 namespace {
 
@@ -22,308 +18,13 @@ constexpr int32_t kMaxPairsLen = 8192;  // 64-bit network elements: 8 KB of SMEM
 constexpr int32_t kMaxLen = 16384;  // 4x the spectra bound of P:L170-173
 
 thread_local int g_last_cuda_error = 0;
-std::atomic<int64_t> g_launches{0};
 
 gas_status cuda_fail(cudaError_t e) {
   g_last_cuda_error = (int)e;
   return GAS_ERROR_CUDA;
 }
 
-int num_sms() {
-  int dev = 0, sms = 0;
-  if (cudaGetDevice(&dev) != cudaSuccess) return 148;
-  if (cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev) != cudaSuccess || sms <= 0) return 148;
-  return sms;
-}
-
-int32_t size_class(int64_t n) {  // smallest power of two >= n, n >= 2
-  int32_t p = 2;
-  while (p < n) p <<= 1;
-  return p;
-}
-
-// Persistent grid: enough blocks to cover the work, at most the number of
-// blocks that can be resident on all SMs at once (a multiple of the SM count).
-// GAS_GRID_CAP=k (testing knob): at most k blocks per persistent launch, so that
-// every block sorts many arrays back to back (tools/sanitize_cases.py).
-int64_t grid_cap() {
-  static const int64_t cap = [] {
-    const char* v = std::getenv("GAS_GRID_CAP");
-    return v ? (int64_t)std::atoll(v) : (int64_t)0;
-  }();
-  return cap;
-}
-
-template <typename K>
-int persistent_grid(K kernel, int threads, int64_t blocks_needed) {
-  int per_sm = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kernel, threads, 0) != cudaSuccess || per_sm <= 0)
-    per_sm = 1;
-  int64_t cap = (int64_t)per_sm * num_sms();
-  if (grid_cap() > 0 && grid_cap() < cap) cap = grid_cap();
-  return (int)(blocks_needed < cap ? (blocks_needed > 0 ? blocks_needed : 1) : cap);
-}
-
-template <typename K>
-int persistent_grid_smem(K kernel, int threads, int smem, int64_t blocks_needed) {
-  int per_sm = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kernel, threads, smem) != cudaSuccess || per_sm <= 0)
-    per_sm = 1;
-  int64_t cap = (int64_t)per_sm * num_sms();
-  if (grid_cap() > 0 && grid_cap() < cap) cap = grid_cap();
-  return (int)(blocks_needed < cap ? (blocks_needed > 0 ? blocks_needed : 1) : cap);
-}
-
-template <int KPT, int G, bool VEC>
-cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  constexpr int blk = gas::warp_block<G>();
-  constexpr int smem = gas::warp_smem_bytes<KPT, G>();
-  constexpr int arrays_per_block = (blk / 32) * (32 / G);
-  auto k = gas::k_fixed_warp<KPT, G, VEC>;
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-  if (e != cudaSuccess) return e;
-  const int grid = persistent_grid_smem(k, blk, smem, (N + arrays_per_block - 1) / arrays_per_block);
-  k<<<grid, blk, smem, s>>>(d, N, n, 1u);
-  return cudaGetLastError();
-}
-
-
-template <int W, int WR, bool VEC>
-cudaError_t launch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  auto k = gas::k_fixed_cta<W, WR, VEC>;
-  constexpr int smem = gas::cta_smem_bytes<W, WR>();
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-  if (e != cudaSuccess) return e;
-  k<<<persistent_grid_smem(k, 32 * WR, smem, N), 32 * WR, smem, s>>>(d, N, n, 1u);
-  return cudaGetLastError();
-}
-
-bool offsets512_bucket() {  // GAS_OFFSETS512=0: the (256, 512] offsets class on the network kernel
-  const char* v = std::getenv("GAS_OFFSETS512");
-  return !(v && std::strcmp(v, "0") == 0);
-}
-
-bool bucket_enabled() {
-  const char* v = std::getenv("GAS_BUCKET");
-  return !(v && std::strcmp(v, "0") == 0);
-}
-
-// Bucket-then-network, one array per CTA of W warps (bucket_cta.cuh).
-template <int W, int WR, bool VEC>
-cudaError_t launch_fixed_bucket_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  auto k = gas::k_fixed_bucket_cta<W, WR, VEC>;
-  constexpr int gr = gas::bkc_groups<WR>(), blk = gas::bkc_block<WR>();
-  constexpr int smem = gas::BkCta<W, WR>::SMEM * gr;
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-  if (e != cudaSuccess) return e;
-  k<<<persistent_grid_smem(k, blk, smem, (N + gr - 1) / gr), blk, smem, s>>>(d, N, n, 1u);
-  return cudaGetLastError();
-}
-
-template <int W, int WR, int RV = 16>
-cudaError_t launch_offsets_bucket(uint32_t* d, const int64_t* off, int64_t N, int64_t lo, int64_t hi,
-                                  unsigned long long* ctr, cudaStream_t s) {
-  auto k = gas::k_offsets_bucket<W, WR, RV>;
-  constexpr int gr = 1, blk = 32 * WR;
-  constexpr int smem = gas::BkCta<W, WR>::SMEM * gr;
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-  if (e != cudaSuccess) return e;
-  k<<<persistent_grid_smem(k, blk, smem, ((N + 31) / 32 + gr - 1) / gr), blk, smem, s>>>(d, off, N, lo, hi, ctr, 1u);
-  return cudaGetLastError();
-}
-
-// Fixed-length CTA classes (n > 1024): W warps' network, WR = ceil(n / 1024) real
-// warps rounded to the instantiated set (padding blocks are virtual, see sort_cta).
-template <bool VEC>
-cudaError_t dispatch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  if (bucket_enabled()) {
-    if (n <= 2048) return launch_fixed_bucket_cta<2, 2, VEC>(d, N, n, s);
-    if (n <= 3072) return launch_fixed_bucket_cta<4, 3, VEC>(d, N, n, s);
-    if (n <= 4096) return launch_fixed_bucket_cta<4, 4, VEC>(d, N, n, s);
-    if (n <= 6144) return launch_fixed_bucket_cta<8, 6, VEC>(d, N, n, s);
-    if (n <= 8192) return launch_fixed_bucket_cta<8, 8, VEC>(d, N, n, s);
-    if (n <= 12288) return launch_fixed_bucket_cta<16, 12, VEC>(d, N, n, s);
-    return launch_fixed_bucket_cta<16, 16, VEC>(d, N, n, s);
-  }
-  if (n <= 2048) return launch_fixed_cta<2, 2, VEC>(d, N, n, s);
-  if (n <= 3072) return launch_fixed_cta<4, 3, VEC>(d, N, n, s);
-  if (n <= 4096) return launch_fixed_cta<4, 4, VEC>(d, N, n, s);
-  if (n <= 6144) return launch_fixed_cta<8, 6, VEC>(d, N, n, s);
-  if (n <= 8192) return launch_fixed_cta<8, 8, VEC>(d, N, n, s);
-  if (n <= 12288) return launch_fixed_cta<16, 12, VEC>(d, N, n, s);
-  return launch_fixed_cta<16, 16, VEC>(d, N, n, s);
-}
-
-bool env_flag(const char* name) {
-  const char* v = std::getenv(name);
-  return v && v[0] != '\0' && std::strcmp(v, "0") != 0;
-}
-
-cudaError_t launch_fixed_1024_tma(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  // per-device attribute: set on every call (cheap), the current device may change
-  const cudaError_t attr = cudaFuncSetAttribute(gas::k_fixed_1024_tma, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                                gas::kTmaSmemBytes);
-  if (attr != cudaSuccess) return attr;
-  int per_sm = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, gas::k_fixed_1024_tma, gas::kWarpBlock,
-                                                    gas::kTmaSmemBytes) != cudaSuccess || per_sm <= 0)
-    per_sm = 1;
-  const int64_t need = (N + gas::kWarpBlock / 32 - 1) / (gas::kWarpBlock / 32);
-  const int64_t cap = (int64_t)per_sm * num_sms();
-  const int grid = (int)(need < cap ? need : cap);
-  gas::k_fixed_1024_tma<<<grid, gas::kWarpBlock, gas::kTmaSmemBytes, s>>>(d, N, n, 1u);
-  return cudaGetLastError();
-}
-
-// Bucket-then-network kernel for 512 < n <= 1024 with aligned rows
-// (bucket1024.cuh). Default on; GAS_BUCKET=0 selects the pure network.
-template <bool VEC>
-cudaError_t launch_fixed_bucket1024(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  auto k = VEC ? gas::k_fixed_bucket1024 : gas::k_fixed_bucket1024_any<false>;
-  const cudaError_t attr = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kBkSmemBytes);
-  if (attr != cudaSuccess) return attr;
-  const int grid = persistent_grid_smem(k, gas::kBkBlock, gas::kBkSmemBytes,
-                                        (N + gas::kBkBlock / 32 - 1) / (gas::kBkBlock / 32));
-  k<<<grid, gas::kBkBlock, gas::kBkSmemBytes, s>>>(d, N, n, 1u);
-  return cudaGetLastError();
-}
-
-// Bucket-then-network kernel for 256 < n <= 512 with aligned rows (bucket512.cuh).
-cudaError_t launch_fixed_bucket512(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  const cudaError_t attr = cudaFuncSetAttribute(gas::k_fixed_bucket512, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                                gas::kBk5SmemBytes);
-  if (attr != cudaSuccess) return attr;
-  const int grid = persistent_grid_smem(gas::k_fixed_bucket512, gas::kBk5Block, gas::kBk5SmemBytes,
-                                        (N + GAS_BK5_WARPS - 1) / GAS_BK5_WARPS);
-  gas::k_fixed_bucket512<<<grid, gas::kBk5Block, gas::kBk5SmemBytes, s>>>(d, N, n, 1u);
-  return cudaGetLastError();
-}
-
-template <bool VEC>
-cudaError_t dispatch_fixed(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  switch (size_class(n)) {
-    case 2: return launch_fixed_warp<2, 1, false>(d, N, n, s);
-    case 4: return launch_fixed_warp<4, 1, VEC>(d, N, n, s);
-    case 8: return launch_fixed_warp<8, 1, VEC>(d, N, n, s);
-    case 16: return launch_fixed_warp<16, 1, VEC>(d, N, n, s);
-    case 32: return launch_fixed_warp<32, 1, VEC>(d, N, n, s);
-    case 64: return launch_fixed_warp<32, 2, VEC>(d, N, n, s);
-    case 128: return launch_fixed_warp<32, 4, VEC>(d, N, n, s);
-    case 256: return launch_fixed_warp<32, 8, VEC>(d, N, n, s);
-    case 512:
-      if (VEC && bucket_enabled()) return launch_fixed_bucket512(d, N, n, s);
-      return launch_fixed_warp<32, 16, VEC>(d, N, n, s);
-    case 1024:
-      // TMA-prefetch variant: opt-in (GAS_TMA=1). Measured on B200 it removes the
-      // global-load stalls but is 5% slower overall (profiles/r01_ab_tma.txt):
-      // the kernel is ALU/issue-bound, not latency-bound.
-      if (VEC && env_flag("GAS_TMA")) return launch_fixed_1024_tma(d, N, n, s);
-      if (bucket_enabled()) return launch_fixed_bucket1024<VEC>(d, N, n, s);
-      return launch_fixed_warp<32, 32, VEC>(d, N, n, s);
-    default: return dispatch_fixed_cta<VEC>(d, N, n, s);
-  }
-  return cudaErrorInvalidValue;
-}
-
-template <int KPT, int G>
-cudaError_t launch_offsets_warp(uint32_t* d, const int64_t* off, int64_t N, cudaStream_t s) {
-  constexpr int blk = gas::warp_block<G>();
-  constexpr int smem = gas::warp_smem_bytes<KPT, G>();
-  auto k = gas::k_offsets_warp<KPT, G>;
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-  if (e != cudaSuccess) return e;
-  const int64_t windows = (N + 31) / 32;
-  const int grid = persistent_grid_smem(k, blk, smem, (windows + blk / 32 - 1) / (blk / 32));
-  k<<<grid, blk, smem, s>>>(d, off, N, 1u);
-  return cudaGetLastError();
-}
-
-template <int W, int WR>
-cudaError_t launch_offsets_cta(uint32_t* d, const int64_t* off, int64_t N, int64_t lo, int64_t hi,
-                               unsigned long long* ctr, cudaStream_t s) {
-  auto k = gas::k_offsets_cta<W, WR>;
-  constexpr int smem = gas::cta_smem_bytes<W, WR>();
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-  if (e != cudaSuccess) return e;
-  k<<<persistent_grid_smem(k, 32 * WR, smem, (N + 31) / 32), 32 * WR, smem, s>>>(d, off, N, lo, hi, ctr, 1u);
-  return cudaGetLastError();
-}
-
-cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, int64_t N, unsigned long long* ctr,
-                                   cudaStream_t s) {
-  switch (P) {
-    case 2: return launch_offsets_warp<2, 1>(d, off, N, s);
-    case 4: return launch_offsets_warp<4, 1>(d, off, N, s);
-    case 8: return launch_offsets_warp<8, 1>(d, off, N, s);
-    case 16: return launch_offsets_warp<16, 1>(d, off, N, s);
-    case 32: return launch_offsets_warp<32, 1>(d, off, N, s);
-    case 64: return launch_offsets_warp<32, 2>(d, off, N, s);
-    case 128: return launch_offsets_warp<32, 4>(d, off, N, s);
-    case 256: return launch_offsets_warp<32, 8>(d, off, N, s);
-    case 512:
-      if (bucket_enabled() && offsets512_bucket()) return launch_offsets_bucket<1, 1, 8>(d, off, N, 256, 512, ctr + 8, s);
-      return launch_offsets_warp<32, 16>(d, off, N, s);
-    case 1024:
-      if (bucket_enabled()) return launch_offsets_bucket<1, 1>(d, off, N, 512, 1024, ctr + 7, s);
-      return launch_offsets_warp<32, 32>(d, off, N, s);
-    case 2048:
-      if (bucket_enabled()) return launch_offsets_bucket<2, 2>(d, off, N, 1024, 2048, ctr, s);
-      return launch_offsets_cta<2, 2>(d, off, N, 1024, 2048, ctr, s);
-    case 3072:
-      if (bucket_enabled()) return launch_offsets_bucket<4, 3>(d, off, N, 2048, 3072, ctr + 1, s);
-      return launch_offsets_cta<4, 3>(d, off, N, 2048, 3072, ctr + 1, s);
-    case 4096:
-      if (bucket_enabled()) return launch_offsets_bucket<4, 4>(d, off, N, 3072, 4096, ctr + 2, s);
-      return launch_offsets_cta<4, 4>(d, off, N, 3072, 4096, ctr + 2, s);
-    case 6144:
-      if (bucket_enabled()) return launch_offsets_bucket<8, 6>(d, off, N, 4096, 6144, ctr + 3, s);
-      return launch_offsets_cta<8, 6>(d, off, N, 4096, 6144, ctr + 3, s);
-    case 8192:
-      if (bucket_enabled()) return launch_offsets_bucket<8, 8>(d, off, N, 6144, 8192, ctr + 4, s);
-      return launch_offsets_cta<8, 8>(d, off, N, 6144, 8192, ctr + 4, s);
-    case 12288:
-      if (bucket_enabled()) return launch_offsets_bucket<16, 12>(d, off, N, 8192, 12288, ctr + 5, s);
-      return launch_offsets_cta<16, 12>(d, off, N, 8192, 12288, ctr + 5, s);
-    case 16384:
-      if (bucket_enabled()) return launch_offsets_bucket<16, 16>(d, off, N, 12288, 16384, ctr + 6, s);
-      return launch_offsets_cta<16, 16>(d, off, N, 12288, 16384, ctr + 6, s);
-  }
-  return cudaErrorInvalidValue;
-}
-
-template <int KPT, int G, int W>
-cudaError_t launch_pairs(uint32_t* k, uint32_t* v, int64_t N, int n, cudaStream_t s) {
-  using C = gas::PairsCfg<KPT, G, W>;
-  auto kern = gas::k_pairs<KPT, G, W>;
-  cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
-  if (e != cudaSuccess) return e;
-  int per_sm = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, C::TPB, C::SMEM) != cudaSuccess || per_sm <= 0)
-    per_sm = 1;
-  const int64_t need = (N + C::GROUPS - 1) / C::GROUPS;
-  const int64_t cap = (int64_t)per_sm * num_sms();
-  kern<<<(int)(need < cap ? need : cap), C::TPB, C::SMEM, s>>>(k, v, N, n);
-  return cudaGetLastError();
-}
-
-cudaError_t dispatch_pairs(uint32_t* k, uint32_t* v, int64_t N, int n, cudaStream_t s) {
-  switch (size_class(n)) {
-    case 2: return launch_pairs<2, 1, 1>(k, v, N, n, s);
-    case 4: return launch_pairs<4, 1, 1>(k, v, N, n, s);
-    case 8: return launch_pairs<8, 1, 1>(k, v, N, n, s);
-    case 16: return launch_pairs<16, 1, 1>(k, v, N, n, s);
-    case 32: return launch_pairs<32, 1, 1>(k, v, N, n, s);
-    case 64: return launch_pairs<32, 2, 1>(k, v, N, n, s);
-    case 128: return launch_pairs<32, 4, 1>(k, v, N, n, s);
-    case 256: return launch_pairs<32, 8, 1>(k, v, N, n, s);
-    case 512: return launch_pairs<32, 16, 1>(k, v, N, n, s);
-    case 1024: return launch_pairs<32, 32, 1>(k, v, N, n, s);
-    case 2048: return launch_pairs<32, 32, 2>(k, v, N, n, s);
-    case 4096: return launch_pairs<32, 32, 4>(k, v, N, n, s);
-    case 8192: return launch_pairs<32, 32, 8>(k, v, N, n, s);
-  }
-  return cudaErrorInvalidValue;
-}
+using namespace gas_host;
 
 // GAS_CHECK=1 validation of CSR offsets: flag = 1 on any violation.
 __global__ void k_check_offsets(const int64_t* __restrict__ off, int64_t N, int64_t max_len, int* flag) {
@@ -435,10 +136,11 @@ gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len,
   if (d_data == nullptr || (reinterpret_cast<uintptr_t>(d_data) & 3u)) return GAS_ERROR_INVALID_VALUE;
   uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
   const bool vec = (reinterpret_cast<uintptr_t>(d_data) & 15u) == 0 && (array_len & 3) == 0;
-  const cudaError_t e = vec ? dispatch_fixed<true>(d, num_arrays, array_len, stream)
-                            : dispatch_fixed<false>(d, num_arrays, array_len, stream);
+  const cudaError_t e = array_len <= 512    ? dispatch_fixed_small(vec, d, num_arrays, array_len, stream)
+                        : array_len <= 1024 ? dispatch_fixed_1024(vec, d, num_arrays, array_len, stream)
+                                            : dispatch_fixed_cta(vec, d, num_arrays, array_len, stream);
   if (e != cudaSuccess) return cuda_fail(e);
-  g_launches.fetch_add(1, std::memory_order_relaxed);
+  if (array_len <= 512 || array_len > 1024) launch_counter() += 1;  // the 1024 class counts its own launches
   return GAS_SUCCESS;
 }
 
@@ -457,7 +159,7 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
     int h = 0;
     cudaMemsetAsync(flag, 0, sizeof(int), stream);
     k_check_offsets<<<num_sms() * 4, 256, 0, stream>>>(d_offsets, num_arrays, max_array_len, flag);
-    g_launches.fetch_add(1, std::memory_order_relaxed);
+    launch_counter() += 1;
     cudaMemcpyAsync(&h, flag, sizeof(int), cudaMemcpyDeviceToHost, stream);
     cudaFreeAsync(flag, stream);
     e = cudaStreamSynchronize(stream);
@@ -493,7 +195,7 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
     for (int c = 0; c < nclass; ++c) {
       const cudaError_t e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, ctr, stream);
       if (e != cudaSuccess) return cuda_fail(e);
-      g_launches.fetch_add(1, std::memory_order_relaxed);
+      launch_counter() += 1;
     }
     return GAS_SUCCESS;
   }
@@ -503,7 +205,7 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
   for (int i = 0; i < K && e == cudaSuccess; ++i) e = cudaStreamWaitEvent(ss->s[i], ss->fork, 0);
   for (int c = nclass - 1, i = 0; c >= 0 && e == cudaSuccess; --c, ++i) {
     e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, ctr, ss->s[i % K]);
-    if (e == cudaSuccess) g_launches.fetch_add(1, std::memory_order_relaxed);
+    if (e == cudaSuccess) launch_counter() += 1;
   }
   // always join (also after an error) so that the caller's stream never races ahead
   for (int i = 0; i < K; ++i) {
@@ -524,7 +226,7 @@ gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays,
     return GAS_ERROR_INVALID_VALUE;
   const cudaError_t e = dispatch_pairs(reinterpret_cast<uint32_t*>(d_keys), d_values, num_arrays, array_len, stream);
   if (e != cudaSuccess) return cuda_fail(e);
-  g_launches.fetch_add(1, std::memory_order_relaxed);
+  launch_counter() += 1;
   return GAS_SUCCESS;
 }
 
@@ -588,6 +290,6 @@ const char* gas_status_string(gas_status s) {
 
 int gas_last_cuda_error(void) { return g_last_cuda_error; }
 
-int64_t gas_launch_count(void) { return g_launches.load(std::memory_order_relaxed); }
+int64_t gas_launch_count(void) { return launch_counter().load(std::memory_order_relaxed); }
 
 }  // extern "C"

@@ -195,7 +195,7 @@ __global__ void __launch_bounds__(warp_block<G>(), warp_block_min<G>()) k_fixed_
 // path. Dynamic shared memory: kWarpBlock/32 warps x 2 x 4 KB + barriers.
 constexpr int kTmaSmemBytes = (kWarpBlock / 32) * 2 * 4096 + (kWarpBlock / 32) * 2 * 8;
 
-__global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS)
+static __global__ void __launch_bounds__(kWarpBlock, GAS_WARP_MIN_BLOCKS)
     k_fixed_1024_tma(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   extern __shared__ __align__(128) uint4 dsm[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
