@@ -226,19 +226,16 @@ __device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
 }
 
 // ---- Control block of the 512 < n <= 1024 pipeline (sort1024.cuh): device
-// workspace of one gas_sort_arrays call, followed by two array-index lists of
-// N entries each.
+// workspace of one gas_sort_arrays call, followed by an array-index list of
+// up to N entries.
 enum : uint32_t { kS1Bucket = 0, kS1Count = 1, kS1Network = 2 };
 struct S1Ctl {
-  uint32_t votes[3];  // sampler: arrays voting for each path
-  uint32_t done;      // sampler blocks finished
-  uint32_t flag;      // the path that takes the whole batch (kS1*)
-  uint32_t n1;        // list 1: arrays the bucket kernel hands to the counting sort
-  uint32_t n2;        // list 2: arrays handed to the network
-  uint32_t pad;
+  uint32_t flag;      // the path that takes the whole batch (kS1*), written by the sampler
+  uint32_t nlist;     // arrays the counting-sort kernel hands to the network (zeroed by the sampler)
 };
-__device__ __forceinline__ uint32_t* s1_list1(S1Ctl* c, int64_t N) { return reinterpret_cast<uint32_t*>(c + 1); }
-__device__ __forceinline__ uint32_t* s1_list2(S1Ctl* c, int64_t N) { return reinterpret_cast<uint32_t*>(c + 1) + N; }
+// The list of nlist array indices follows the control block.
+__device__ __forceinline__ uint32_t* s1_list(S1Ctl* c) { return reinterpret_cast<uint32_t*>(c + 1); }
+__device__ __forceinline__ const uint32_t* s1_list(const S1Ctl* c) { return reinterpret_cast<const uint32_t*>(c + 1); }
 __device__ __forceinline__ void s1_push(uint32_t& count, uint32_t* list, int64_t a, int lane) {
   if (lane == 0) list[atomicAdd(&count, 1u)] = (uint32_t)a;
 }
@@ -267,16 +264,19 @@ __device__ __forceinline__ uint32_t bk_sample_key(const uint32_t (&k)[32], int l
   }
 }
 
-// Overflow predictor of the value buckets: the 32-key sample k0 (one key per
-// lane) must not put >= 12 keys into the 8 lowest or the 8 highest buckets
-// (all-positive arrays: peaked values such as log-normal intensities), nor
-// >= GAS_S1_PRED keys into one bucket (other arrays: duplicates, zeros).
+// Overflow predictor of the value buckets (the pipeline's sampler and the
+// fused small-batch kernel): the 32-key sample k0 (one key per lane) must not
+// put >= 12 keys into the 8 lowest or the 8 highest buckets (peaked values
+// such as log-normal intensities), >= GAS_S1_PRED keys into one bucket, or
+// repeat one value >= 3 times (duplicate-heavy arrays: a repeated value fills
+// a bucket no map can split).
 __device__ __forceinline__ bool bk_sample_ok(uint32_t k0, bool raw, float vmin, float s) {
   const uint32_t sb = bucket_bits(k0, vmin, s) - 0x4B000000u;
-  if (raw)
-    return __popc(__ballot_sync(0xffffffffu, sb < 8u)) < 12 &&
-           __popc(__ballot_sync(0xffffffffu, sb > (uint32_t)GAS_BK_TOP - 8u)) < 12;
-  return __reduce_max_sync(0xffffffffu, __popc(__match_any_sync(0xffffffffu, sb))) < GAS_S1_PRED;
+  const bool skew = __popc(__ballot_sync(0xffffffffu, sb < 8u)) >= 12 ||
+                    __popc(__ballot_sync(0xffffffffu, sb > (uint32_t)GAS_BK_TOP - 8u)) >= 12;
+  const int bmax = __reduce_max_sync(0xffffffffu, __popc(__match_any_sync(0xffffffffu, sb)));
+  const int vmax = __reduce_max_sync(0xffffffffu, __popc(__match_any_sync(0xffffffffu, k0)));
+  return !skew && bmax < GAS_S1_PRED && vmax < 3;
 }
 
 // Fixed-length arrays, 512 < n <= 1024, 16-byte-aligned rows (n % 4 == 0).
@@ -300,8 +300,10 @@ __device__ __forceinline__ bool bk_sample_ok(uint32_t k0, bool raw, float vmin, 
 //     first size_b network outputs are bucket b sorted in both rounds.
 //     Outputs are staged at slot words kBkStageWord + base_b + i.
 //  5. coalesced in-place store (key -> bits for non-raw arrays).
-static __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
-    k_fixed_bucket1024(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one, S1Ctl* ctl) {
+template <bool PIPE>
+__global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
+    k_fixed_bucket1024(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one, const S1Ctl* ctl) {
+  if (PIPE && ctl->flag != kS1Bucket) return;  // pipeline (sort1024.cuh): another kernel takes this batch
   extern __shared__ __align__(16) uint4 bk_smem[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
@@ -316,7 +318,6 @@ static __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kB
   const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;  // counter address = bucket bits * 4 + cnt_b0
   const uint32_t row0 = slot_sa + lane * (kBkRowWords * 4);  // this lane's rows: buckets lane, lane + 32
   const uint32_t row1 = row0 + 32 * (kBkRowWords * 4);
-  if (ctl && ctl->flag != kS1Bucket) return;  // pipeline: another kernel takes this batch
 
   for (int64_t a = (int64_t)blockIdx.x * (kBkBlock / 32) + warp; a < N; a += nwarps) {
     uint4* const dst = reinterpret_cast<uint4*>(d + a * (int64_t)n);
@@ -369,9 +370,6 @@ static __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kB
     const float range = __fsub_rn(vmax, vmin);
     const float s = __fdiv_rn((float)GAS_BK_TOP, range);
     use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
-    // pipeline mode (sort1024.cuh): arrays the 32-key sample predicts to
-    // overflow go to the counting sort without a bucket attempt
-    if (ctl && use_buckets) use_buckets = bk_sample_ok(bk_sample_key<true>(k, lane), raw, vmin, s);
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
     if (use_buckets) {
       // lane l owns buckets l (row l) and l + 32 (row 32 + l)
@@ -463,8 +461,6 @@ static __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kB
           stg_cs_if(q < 4 || c < nc, dst + c, v);
         }
       }
-    } else if (ctl) {  // pipeline: the counting-sort kernel takes this array
-      s1_push(ctl->n1, s1_list1(ctl, N), a, lane);
     } else {
       __syncwarp();  // the fallback's scratch overlaps the slot buffer
       bucket1024_fallback(k, dst, nc, lane, slot_ptr, one);
@@ -478,9 +474,10 @@ static __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kB
 // lane + 32 r (4-byte accesses). Kept apart from k_fixed_bucket1024 so that the
 // 16-byte kernel's register allocation stays as measured (a merged template
 // spilled 12 bytes per array: 4.21 -> 4.31 ms).
-template <bool VEC>
+template <bool VEC, bool PIPE>
 __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
-    k_fixed_bucket1024_any(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one, S1Ctl* ctl) {
+    k_fixed_bucket1024_any(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one, const S1Ctl* ctl) {
+  if (PIPE && ctl->flag != kS1Bucket) return;  // pipeline (sort1024.cuh): another kernel takes this batch
   extern __shared__ __align__(16) uint4 bk_smem[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
@@ -495,7 +492,6 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
   const uint32_t cnt_b0 = cnt_sa - 0x4B000000u * 4u;  // counter address = bucket bits * 4 + cnt_b0
   const uint32_t row0 = slot_sa + lane * (kBkRowWords * 4);  // this lane's rows: buckets lane, lane + 32
   const uint32_t row1 = row0 + 32 * (kBkRowWords * 4);
-  if (ctl && ctl->flag != kS1Bucket) return;  // pipeline: another kernel takes this batch
 
   // key r of this lane lies inside the array (always for r < 16: n > 512)
   auto valid = [&](int r) -> bool {
@@ -558,9 +554,6 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     const float range = __fsub_rn(vmax, vmin);
     const float s = __fdiv_rn((float)GAS_BK_TOP, range);
     use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
-    // pipeline mode (sort1024.cuh): arrays the 32-key sample predicts to
-    // overflow go to the counting sort without a bucket attempt
-    if (ctl && use_buckets) use_buckets = bk_sample_ok(bk_sample_key<VEC>(k, lane), raw, vmin, s);
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
     if (use_buckets) {
       // lane l owns buckets l (row l) and l + 32 (row 32 + l)
@@ -662,8 +655,6 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
           stg_cs_if(q < 4 || c < nc, dst + c, v);
         }
       }
-    } else if (ctl) {  // pipeline: the counting-sort kernel takes this array
-      s1_push(ctl->n1, s1_list1(ctl, N), a, lane);
     } else {
       __syncwarp();  // the fallback's scratch overlaps the slot buffer
       if constexpr (VEC) bucket1024_fallback(k, dst, nc, lane, slot_ptr, one);

@@ -46,7 +46,7 @@ cudaError_t launch_fixed_1024_tma(uint32_t* d, int64_t N, int n, cudaStream_t s)
 // (bucket1024.cuh). Default on; GAS_BUCKET=0 selects the pure network.
 template <bool VEC>
 cudaError_t launch_fixed_bucket1024(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  auto k = VEC ? gas::k_fixed_bucket1024 : gas::k_fixed_bucket1024_any<false>;
+  auto k = VEC ? gas::k_fixed_bucket1024<false> : gas::k_fixed_bucket1024_any<false, false>;
   const cudaError_t attr = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kBkSmemBytes);
   if (attr != cudaSuccess) return attr;
   const int grid = persistent_grid_smem(k, gas::kBkBlock, gas::kBkSmemBytes,
@@ -74,20 +74,17 @@ cudaError_t launch_fixed_sort1024(uint32_t* d, int64_t N, int n, cudaStream_t s)
 
 // Default for large batches: the device-routed pipeline of sort1024.cuh
 // (sampler -> bucket kernel -> counting-sort kernel -> network kernel), 4
-// launches and 8 N + 32 bytes of stream-ordered workspace.
+// launches and 4 N + 8 bytes of stream-ordered workspace.
 template <bool VEC>
 cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   void* ws = nullptr;
-  cudaError_t e = ws_alloc(&ws, sizeof(gas::S1Ctl) + 8 * (size_t)N, s);
+  cudaError_t e = ws_alloc(&ws, sizeof(gas::S1Ctl) + 4 * (size_t)N, s);
   if (e != cudaSuccess) return e;
   gas::S1Ctl* ctl = static_cast<gas::S1Ctl*>(ws);
-  e = cudaMemsetAsync(ctl, 0, sizeof(gas::S1Ctl), s);
+  gas::k_s1_sample<VEC><<<1, 1024, 0, s>>>(d, N, n, ctl);
+  e = cudaGetLastError();
   if (e == cudaSuccess) {
-    gas::k_s1_sample<VEC><<<4, 512, 0, s>>>(d, N, n, ctl);
-    e = cudaGetLastError();
-  }
-  if (e == cudaSuccess) {
-    auto k = VEC ? gas::k_fixed_bucket1024 : gas::k_fixed_bucket1024_any<false>;
+    auto k = VEC ? gas::k_fixed_bucket1024<true> : gas::k_fixed_bucket1024_any<false, true>;
     e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kBkSmemBytes);
     if (e == cudaSuccess) {
       const int grid = persistent_grid_smem(k, gas::kBkBlock, gas::kBkSmemBytes,

@@ -248,20 +248,18 @@ __global__ void __launch_bounds__(kS1Block, 1)
 // samples when arrays of one batch alternate between the counting sort and
 // the network). So each path is its own kernel, and the batch's work is
 // routed on the device, with no host synchronisation:
-//   1. k_s1_sample: 64 warps load 64 arrays spread over the batch and vote
+//   1. k_s1_sample: 32 warps load 32 arrays spread over the batch and vote
 //      for the path each would take (the same tests as the kernels below);
-//      the last block writes the majority into ctl->flag.
-//   2. k_fixed_bucket1024 (bucket1024.cuh): runs the batch when flag ==
-//      bucket; arrays its sample predicts to overflow, arrays with NaN / inf
-//      and actual overflows go to list 1.
-//   3. k_s1_count: the counting sort over the whole batch (flag == count) or
-//      over list 1; special-heavy arrays go to list 2; arrays failing its own
-//      check are finished by the network inline (rare).
+//      the majority goes to ctl->flag.
+//   2. k_fixed_bucket1024<PIPE = true> (bucket1024.cuh): runs the batch when
+//      flag == bucket, unchanged from the stand-alone kernel (its few
+//      overflowing / NaN arrays take its inline network).
+//   3. k_s1_count: the counting sort over the whole batch when flag == count;
+//      special-heavy arrays go to a list; arrays failing its own check are
+//      finished by the network inline (rare).
 //   4. k_s1_net: the 1024-key network over the whole batch (flag == network)
-//      or over list 2.
-// Kernels not chosen exit at once (a few microseconds each). Arrays that leave
-// the chosen kernel are read from HBM a second time (4 KB each); in the
-// measured distributions that is 0-0.5% of the arrays.
+//      or over that list (its arrays are read from HBM a second time).
+// Kernels not chosen exit at once (a few microseconds each).
 
 // The class an array votes for: special-heavy sample -> network; finite values
 // whose 32-key sample fits the buckets -> bucket; else the counting sort.
@@ -270,13 +268,17 @@ __device__ __forceinline__ uint32_t s1_sample_special(uint32_t k0) {
   return __popc(__ballot_sync(0xffffffffu, special));
 }
 
+// One block of 32 warps; warp w samples array floor(w N / 32). The block
+// writes the majority vote into ctl->flag and zeroes the list counter (no
+// other initialisation of the workspace is needed).
 template <bool VEC>
-__global__ void __launch_bounds__(512, 1) k_s1_sample(const uint32_t* __restrict__ d, int64_t N, int n, S1Ctl* ctl) {
-  const int lane = threadIdx.x & 31;
-  const int w = blockIdx.x * (blockDim.x / 32) + (threadIdx.x >> 5);
-  const int S = gridDim.x * (blockDim.x / 32);
-  if (w < S && (int64_t)w < N) {
-    const int64_t a = (N <= S) ? w : (int64_t)(((__int128)w * N) / S);
+__global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restrict__ d, int64_t N, int n, S1Ctl* ctl) {
+  __shared__ uint32_t votes[3];
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  if (threadIdx.x < 3) votes[threadIdx.x] = 0;
+  __syncthreads();
+  if ((int64_t)w < N) {
+    const int64_t a = (N <= 32) ? w : (int64_t)(((__int128)w * N) >> 5);
     const uint32_t* arr = d + a * (int64_t)n;
     uint32_t k[32];
 #pragma unroll
@@ -312,17 +314,13 @@ __global__ void __launch_bounds__(512, 1) k_s1_sample(const uint32_t* __restrict
       if (ok) ok = bk_sample_ok(bk_sample_key<VEC>(k, lane), raw, vmin, s);
       cls = ok ? kS1Bucket : kS1Count;
     }
-    if (lane == 0) atomicAdd(&ctl->votes[cls], 1u);
+    if (lane == 0) atomicAdd(&votes[cls], 1u);
   }
   __syncthreads();
   if (threadIdx.x == 0) {
-    __threadfence();
-    if (atomicAdd(&ctl->done, 1u) == gridDim.x - 1) {  // the last block decides
-      __threadfence();
-      const uint32_t vb = atomicAdd(&ctl->votes[kS1Bucket], 0u), vc = atomicAdd(&ctl->votes[kS1Count], 0u),
-                     vn = atomicAdd(&ctl->votes[kS1Network], 0u);
-      ctl->flag = (vb >= vc && vb >= vn) ? kS1Bucket : (vc >= vn ? kS1Count : kS1Network);
-    }
+    const uint32_t vb = votes[kS1Bucket], vc = votes[kS1Count], vn = votes[kS1Network];
+    ctl->flag = (vb >= vc && vb >= vn) ? kS1Bucket : (vc >= vn ? kS1Count : kS1Network);
+    ctl->nlist = 0;
   }
 }
 
@@ -346,29 +344,24 @@ __device__ __forceinline__ void s1_load(uint32_t (&k)[32], const uint32_t* arr, 
   for (int r = 16; r < 32; ++r) k[r] = cw_valid<VEC>(r, lane, n) ? k[r] : k[0];
 }
 
-// 3. The counting sort (cw1024.cuh) over the whole batch or over list 1.
+// 3. The counting sort (cw1024.cuh) over the whole batch (flag == count).
 template <bool VEC>
 __global__ void __launch_bounds__(kCwBlock, 1) k_s1_count(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one,
                                                           S1Ctl* ctl) {
   extern __shared__ __align__(16) uint4 cw_smem[];
-  const uint32_t flag = ctl->flag;
-  if (flag == kS1Network) return;
-  const int64_t count = flag == kS1Count ? N : (int64_t)ctl->n1;
-  const uint32_t* list = s1_list1(ctl, N);
+  if (ctl->flag != kS1Count) return;
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t cnt_sa = (uint32_t)__cvta_generic_to_shared(cw_smem) + warp * kCwWarpBytes;
   const uint32_t buf_sa = cnt_sa + kCwCntBytes;
   uint32_t* const buf_ptr =
       reinterpret_cast<uint32_t*>(reinterpret_cast<unsigned char*>(cw_smem) + warp * kCwWarpBytes + kCwCntBytes);
   const int64_t nwarps = (int64_t)gridDim.x * (kCwBlock / 32);
-  for (int64_t i = (int64_t)blockIdx.x * (kCwBlock / 32) + warp; i < count; i += nwarps) {
-    const int64_t a = flag == kS1Count ? i : (int64_t)list[i];
+  for (int64_t a = (int64_t)blockIdx.x * (kCwBlock / 32) + warp; a < N; a += nwarps) {
     uint32_t* const arr = d + a * (int64_t)n;
     uint32_t k[32];
     s1_load<VEC>(k, arr, n, lane);
 #if GAS_BK_PREFETCH
-    if (flag == kS1Count && lane == 0 && i + nwarps < count)
-      prefetch_l2(d + (i + nwarps) * (int64_t)n, n);
+    if (lane == 0 && a + nwarps < N) prefetch_l2(d + (a + nwarps) * (int64_t)n, n);
 #endif
     uint32_t umin = k[0], umax = k[0];
 #pragma unroll
@@ -380,22 +373,23 @@ __global__ void __launch_bounds__(kCwBlock, 1) k_s1_count(uint32_t* __restrict__
     umax = __reduce_max_sync(0xffffffffu, max(umax, k[31]));
     const bool raw = umin > 0u && umax < 0x7F800000u;
     if (!raw && s1_sample_special(bk_sample_key<VEC>(k, lane)) >= 2) {
-      s1_push(ctl->n2, s1_list2(ctl, N), a, lane);
+      s1_push(ctl->nlist, s1_list(ctl), a, lane);  // special-heavy: the network kernel takes it
       continue;
     }
     cw_sort_warp<VEC>(k, raw, umin, umax, 0u, arr, n, lane, cnt_sa, buf_sa, buf_ptr, one);
   }
 }
 
-// 4. The 1024-key network (warp1024.cuh) over the whole batch or over list 2.
+// 4. The 1024-key network (warp1024.cuh) over the whole batch (flag ==
+// network) or over the counting-sort kernel's list.
 constexpr int kS1NetBlock = 512;  // 16 warps per SM at <= 128 registers (the network's best)
 template <bool VEC>
 __global__ void __launch_bounds__(kS1NetBlock, 1) k_s1_net(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one,
                                                            S1Ctl* ctl) {
   extern __shared__ __align__(16) uint4 net_smem[];
   const uint32_t flag = ctl->flag;
-  const int64_t count = flag == kS1Network ? N : (int64_t)ctl->n2;
-  const uint32_t* list = s1_list2(ctl, N);
+  const int64_t count = flag == kS1Network ? N : (int64_t)ctl->nlist;
+  const uint32_t* list = s1_list(ctl);
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   uint32_t* const scratch = reinterpret_cast<uint32_t*>(net_smem) + warp * 1024;
   const int64_t nwarps = (int64_t)gridDim.x * (kS1NetBlock / 32);
