@@ -54,6 +54,11 @@ def parse():
     p.add_argument("--dist-backend", default="nccl", choices=["nccl", "gloo"],
                    help="process-group backend under torchrun (gloo: several ranks may share one GPU, for testing)")
     p.add_argument("--cpu-seconds", type=float, default=10.0, help="target CPU time of the oracle sample")
+    p.add_argument("--scaling", default="auto", choices=["auto", "weak", "strong"],
+                   help="multi-GPU split: weak = every rank sorts N arrays of its own; strong = the config's N "
+                        "arrays are split over the ranks (auto: strong for configs[2], weak otherwise)")
+    p.add_argument("--variant", default="keys", choices=["keys", "pairs"],
+                   help="pairs: gas_sort_pairs (stable key + uint32 payload, 16n bytes per array)")
     return p.parse_args()
 
 
@@ -184,6 +189,18 @@ def cpu_cores():
         return os.cpu_count() or 1
 
 
+def cpu_model():
+    try:
+        with open("/proc/cpuinfo") as f:
+            for line in f:
+                if line.startswith("model name"):
+                    return line.split(":", 1)[1].strip()
+    except Exception:
+        pass
+    import platform
+    return platform.processor() or platform.machine()
+
+
 def run_oracle_sample(cfg, dist, seed, target_s, i0=0):
     """The oracle, as it stands, on all host cores over a bounded sample."""
     import numpy as np
@@ -201,6 +218,7 @@ def run_oracle_sample(cfg, dist, seed, target_s, i0=0):
         t0 = time.perf_counter()
         oracle.sort_arrays_offsets_(data, off)
         rate1 = probe / (time.perf_counter() - t0)  # single thread
+        run_oracle_sample.rate1 = rate1
         S = int(min(cfg["N"], max(probe, rate1 * cores * target_s)))
         off = datagen.offsets_from_lengths(lens_all[:S])
         data = datagen.ragged(dist, seed, 0, off)
@@ -224,6 +242,7 @@ def run_oracle_sample(cfg, dist, seed, target_s, i0=0):
     t0 = time.perf_counter()
     oracle.sort_arrays_(a, threads=1)
     rate1 = probe / (time.perf_counter() - t0)
+    run_oracle_sample.rate1 = rate1
     S = int(min(cfg["N"], max(probe, rate1 * cores * target_s)))
     a = datagen.fixed(dist, seed, i0, S, n)
     t0 = time.perf_counter()
@@ -255,7 +274,8 @@ def reference_arm(args, cfg, dist, seed):
         "vs_baseline": None, "dtype": "f32 (sorted as u32 totalOrder keys)", "data": "synthetic",
         "config": {"workload": cfg["name"], "dist": dist, "array_len": cfg["n"], "seed": seed},
         "cpu_baseline": {"value": value, "unit": "arrays/s", "cores": cores, "kind": "oracle",
-                         "sample": sample, "gbs": value * n_avg * 8 / 1e9},
+                         "sample": sample, "gbs": value * n_avg * 8 / 1e9,
+                         "value_1core": getattr(run_oracle_sample, "rate1", None), "cpu_model": cpu_model()},
         "e2e": {"value": value, "unit": "arrays/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
     print(json.dumps(line), flush=True)
@@ -311,13 +331,24 @@ def main():
 
     from paper_conf_icppw_awans16_b200 import shard
 
-    N_rank = cfg["N"]
-    i0, _ = shard.weak_range(N_rank, rank)  # weak scaling: rank r owns arrays [r*N, (r+1)*N)
+    scaling = args.scaling if args.scaling != "auto" else ("strong" if args.config == 2 else "weak")
     stream = torch.cuda.current_stream()
     ragged = cfg["n"] is None
+    pairs = args.variant == "pairs"
+    if pairs and ragged:
+        raise SystemExit("--variant pairs needs a fixed-length config")
     if ragged:
         import numpy as np
-        lens = datagen.lengths(seed, i0, N_rank, cfg["lo"], cfg["hi"])
+        if scaling == "strong":  # one batch of N arrays split at element-count quantiles
+            lens_all = datagen.lengths(seed, 0, cfg["N"], cfg["lo"], cfg["hi"])
+            off_all = datagen.offsets_from_lengths(lens_all)
+            i0, i1 = shard.offsets_shard(off_all, rank, world)
+            N_rank = i1 - i0
+            lens = lens_all[i0:i1]
+        else:
+            N_rank = cfg["N"]
+            i0, _ = shard.weak_range(N_rank, rank)  # weak scaling: rank r owns arrays [r*N, (r+1)*N)
+            lens = datagen.lengths(seed, i0, N_rank, cfg["lo"], cfg["hi"])
         off_h = datagen.offsets_from_lengths(lens)
         total = int(off_h[-1])
         off_d = torch.from_numpy(off_h).to(dev)
@@ -325,27 +356,48 @@ def main():
         datagen.ragged_device(pristine, off_d, dist, seed, i0, N_rank, stream.cuda_stream)
         alg_bytes = 8 * total + 16 * N_rank
         kernel_hint = "k_offsets"
-        n_desc = f"lengths U{{{cfg['lo']}..{cfg['hi']}}}, mean {total / N_rank:.1f}"
+        n_desc = f"lengths U{{{cfg['lo']}..{cfg['hi']}}}, mean {total / max(1, N_rank):.1f}"
     else:
         n = cfg["n"]
+        if scaling == "strong":
+            i0, i1 = shard.shard_range(cfg["N"], rank, world)
+            N_rank = i1 - i0
+        else:
+            N_rank = cfg["N"]
+            i0, _ = shard.weak_range(N_rank, rank)
         pristine = torch.empty(N_rank, n, dtype=torch.float32, device=dev)
         datagen.fixed_device(pristine, dist, seed, i0, N_rank, n, stream.cuda_stream)
-        alg_bytes = 8 * N_rank * n
-        if 512 < n <= 1024 and n % 4 == 0 and os.environ.get("GAS_BUCKET", "1") != "0":
-            kernel_hint = "k_fixed_bucket1024"  # bucket-then-network kernel (aligned rows)
+        alg_bytes = (16 if pairs else 8) * N_rank * n
+        if pairs:
+            kernel_hint = "k_pairs"
+        elif 512 < n <= 1024 and os.environ.get("GAS_BUCKET", "1") != "0":
+            # the sort1024 pipeline's kernel that takes a batch of this distribution (tools/launches.sh)
+            kernel_hint = {"uniform_bits": "k_s1_count", "spectra_intensity": "k_s1_count", "dup16": "k_s1_count",
+                           "special_mix": "k_s1_net"}.get(dist, "k_fixed_bucket1024")
         else:
             kernel_hint = "k_fixed_warp" if n <= 1024 else "k_fixed_cta"
         n_desc = str(n)
     work = torch.empty_like(pristine)
+    if pairs:  # payload = original position (the spectra use case: (m/z, intensity) pairs)
+        vals_pristine = torch.arange(N_rank * cfg["n"], dtype=torch.int64, device=dev).remainder(cfg["n"]) \
+            .to(torch.int32).view(N_rank, cfg["n"])
+        vals = torch.empty_like(vals_pristine)
 
     def step():
         if ragged:
             gas.gas_sort_arrays_offsets(work, off_d, cfg["hi"])
+        elif pairs:
+            gas.gas_sort_pairs(work, vals)
         else:
             gas.gas_sort_arrays(work)
 
-    for _ in range(args.warmup):
+    def restore():
         work.copy_(pristine)
+        if pairs:
+            vals.copy_(vals_pristine)
+
+    for _ in range(args.warmup):
+        restore()
         step()
     torch.cuda.synchronize()
 
@@ -357,7 +409,7 @@ def main():
         launches0 = gas.launch_count()
         t_wall0 = time.perf_counter()
         for s in range(args.steps):
-            work.copy_(pristine)  # untimed restore: the sort is in place
+            restore()  # untimed restore: the sort is in place
             evs[s][0].record(stream)
             step()
             evs[s][1].record(stream)
@@ -368,14 +420,23 @@ def main():
     per_step = [a.elapsed_time(b) for a, b in evs]
     t_sum = shard.max_over_ranks(sum(per_step), red_dev)  # the slowest rank defines the job
     ms_per_step = t_sum / args.steps
-    total_arrays = N_rank * world
+    rank_ms = [sum(per_step) / args.steps]
+    if pg and world > 1:  # every rank's own time and bandwidth (after the timed region)
+        t = torch.tensor([rank_ms[0], float(alg_bytes)], dtype=torch.float64, device=red_dev)
+        ts = [torch.zeros_like(t) for _ in range(world)]
+        pg.all_gather(ts, t)
+        rank_ms = [float(x[0]) for x in ts]
+        rank_bytes = [float(x[1]) for x in ts]
+    else:
+        rank_bytes = [float(alg_bytes)]
+    total_arrays = cfg["N"] if scaling == "strong" else N_rank * world
     value = total_arrays / (ms_per_step * 1e-3)
     achieved_gbs = alg_bytes / (ms_per_step * 1e-3) / 1e9  # per GPU, per launch (one launch per step)
     peak, peak_src = measured_peak_hbm()
 
     # self-check of the result (not timed): every row nondecreasing in totalOrder
     ok = None
-    if not ragged:
+    if not ragged and not pairs:
         ok = True
         for lo in range(0, N_rank, 200000):
             b = work[lo:lo + 200000].view(torch.int32).to(torch.int64) & 0xFFFFFFFF
@@ -383,32 +444,38 @@ def main():
             ok &= bool((k[:, 1:] >= k[:, :-1]).all())
         del b, k
 
-    # e2e through the host-buffer C-ABI entry point (pinned memory; copies inside the timed region)
+    # e2e through the host-buffer C-ABI entry points (pinned memory; copies inside the timed region)
     e2e = None
-    if not args.no_e2e and not ragged:
-        host = torch.empty(N_rank, cfg["n"], dtype=torch.float32, pin_memory=True)
+    if not args.no_e2e and not pairs:
         host_pristine = pristine.cpu()
+        host = torch.empty(host_pristine.shape, dtype=torch.float32, pin_memory=True)
+        off_host = torch.from_numpy(off_h) if ragged else None
         ts = []
         for s in range(1 + args.e2e_steps):
             host.copy_(host_pristine)
             barrier()
             t0 = time.perf_counter()
-            gas.gas_sort_arrays_host(host)
+            if ragged:
+                gas.gas_sort_arrays_offsets_host(host, off_host, cfg["hi"])
+            else:
+                gas.gas_sort_arrays_host(host)
             dt = time.perf_counter() - t0
             if s > 0:
                 ts.append(dt)
         dt = shard.max_over_ranks(sum(ts), red_dev) / len(ts)
-        nbytes = N_rank * cfg["n"] * 4
+        nbytes = pristine.numel() * 4 + (8 * (N_rank + 1) if ragged else 0)
         e2e = {"value": total_arrays / dt, "unit": "arrays/s", "h2d_bytes_per_step": nbytes,
-               "d2h_bytes_per_step": nbytes, "ms_per_step": dt * 1e3,
-               "api": "gas_sort_arrays_host (pinned host buffer, chunked H2D/sort/D2H overlap)"}
+               "d2h_bytes_per_step": pristine.numel() * 4, "ms_per_step": dt * 1e3,
+               "api": ("gas_sort_arrays_offsets_host" if ragged else "gas_sort_arrays_host")
+               + " (pinned host buffer, chunked H2D/sort/D2H overlap)"}
         del host, host_pristine
 
     cpu = None
-    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+    if rank == 0 and world == 1 and not args.no_cpu_baseline and not pairs:
         v, cores, sample, dt = run_oracle_sample(cfg, dist, seed, args.cpu_seconds)
         cpu = {"value": v, "unit": "arrays/s", "cores": cores, "kind": "oracle", "sample": sample,
-               "seconds": round(dt, 2)}
+               "seconds": round(dt, 2), "value_1core": getattr(run_oracle_sample, "rate1", None),
+               "cpu_model": cpu_model()}
         # the oracle's sorted sample doubles as a bit-exact check of the GPU result on those arrays
         import numpy as np
         ref, ref_off = run_oracle_sample.last
@@ -421,23 +488,28 @@ def main():
     if rank == 0:
         line = {
             "metric": METRIC, "value": value, "unit": "arrays/s", "n_gpus": world, "steps": args.steps,
-            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": "weak",
+            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": scaling,
             "vs_baseline": None, "dtype": "u32 (float32 bit patterns as IEEE totalOrder keys)",
             "data": "synthetic",
-            "config": {"workload": cfg["name"], "num_arrays_per_gpu": N_rank, "array_len": n_desc, "dist": dist,
+            "config": {"workload": cfg["name"] + (" [gas_sort_pairs: key + uint32 payload]" if pairs else ""),
+                       "num_arrays_per_gpu": N_rank, "num_arrays_total": total_arrays, "array_len": n_desc, "dist": dist,
                        "seed": seed, "l2": f"inputs ({pristine.numel() * 4 / 1e9:.2f} GB per GPU) "
                                   + ("larger than" if pristine.numel() * 4 > 126e6 else "SMALLER than (L2-resident)")
                                   + " the 126 MB L2; restored from a pristine copy (untimed) before every step",
-                       "parallelism": f"array-index shards x{world}, no collective"},
+                       "parallelism": f"array-index shards x{world} ({scaling} scaling), no collective"},
             "gbs_per_gpu": achieved_gbs,
+            "per_rank": {"ms_per_step": rank_ms, "gbs": [b / (m * 1e-3) / 1e9 for b, m in zip(rank_bytes, rank_ms)]},
             "roofline": {"bound": "hbm", "achieved": achieved_gbs, "peak": peak, "unit": "GB/s",
                          "frac": achieved_gbs / peak, "traffic": ncu_traffic(kernel_hint),
                          "peak_source": peak_src, "kernel": kernel_hint,
-                         "algorithmic_bytes_per_launch": alg_bytes},
-            "issue_roofline": (issue_roofline(kernel_hint, value / world, clk.summary()["sm_mhz"],
+                         "algorithmic_bytes_per_launch": alg_bytes,
+                         "timed": "the whole C-ABI call per step (CUDA events on its stream); for 512 < n <= 1024 "
+                                  "and N >= 16384 that is the sort1024 pipeline's 4 launches, the kernel named "
+                                  "plus ~20 us of sampler / idle-path launches (profiles/ launch lists)"},
+            "issue_roofline": (issue_roofline(kernel_hint, N_rank / (ms_per_step * 1e-3), clk.summary()["sm_mhz"],
                                               torch.cuda.get_device_properties(dev).multi_processor_count)
                                if not ragged and cfg["n"] == 1000 else None),
-            "smem_roofline": (smem_roofline(kernel_hint, value / world, clk.summary()["sm_mhz"],
+            "smem_roofline": (smem_roofline(kernel_hint, N_rank / (ms_per_step * 1e-3), clk.summary()["sm_mhz"],
                                             torch.cuda.get_device_properties(dev).multi_processor_count)
                               if not ragged and cfg["n"] == 1000 else None),
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches,

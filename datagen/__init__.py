@@ -4,7 +4,7 @@ This module holds none of the sort's arithmetic: it only turns a counter
 hash of (seed, array i, position j) into float32 bit patterns.  The recipe is
 written out in ``datagen/gasgen.h``; this file is the numpy twin of the device
 generator ``datagen/gasgen.cu`` (built into ``datagen/libgasgen.so``), and the
-two agree bit for bit (tests/test_datagen_gpu.py).
+two agree bit for bit (tests/test_gpu_parity.py::test_device_generator_matches_numpy).
 
 The workloads follow PAPER.md §7.2 (arrays of
 n = 1000..4000 float32 "uniformly distributed between 0 and 2^31 - 1") and

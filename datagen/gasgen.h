@@ -5,7 +5,8 @@
  * CUDA path and the CPU oracle take their inputs from. It holds none of the
  * sort's arithmetic: it only produces float32 bit patterns from a counter
  * hash. The numpy twin is datagen/__init__.py; both implement exactly the
- * recipe below, bit for bit (checked by tests/test_datagen_gpu.py).
+ *  recipe below, bit for bit (checked by
+ * tests/test_gpu_parity.py::test_device_generator_matches_numpy).
  *
  * Recipe:
  *   mix(z)  = splitmix64 finalizer:

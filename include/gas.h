@@ -19,9 +19,13 @@
  *
  * Conventions for every entry point:
  *   - Pointers named d_* are DEVICE memory of the current device, owned by
- *     the caller; gas_sort_arrays and gas_sort_pairs allocate nothing (zero
- *     workspace); the offsets variant keeps 72 bytes and 8 side streams per stream (see there); the library
- *     never calls cudaSetDevice.
+ *     the caller; the library never calls cudaSetDevice. Workspace, where an
+ *     entry point needs any, is stream-ordered (allocated and freed on
+ *     `stream`) from a library-owned memory pool per device that keeps its
+ *     memory, so steady-state calls never allocate from the driver and never
+ *     synchronise: gas_sort_arrays with 512 < array_len <= 1024 and
+ *     num_arrays >= 16384, 4 * num_arrays + 8 bytes; gas_sort_arrays_offsets
+ *     with max_array_len > 256, 72 bytes. Everything else: zero workspace.
  *   - Work is enqueued on `stream` (0 = legacy default stream) and the call
  *     returns without a host synchronisation. Argument and launch-
  *     configuration errors are returned synchronously; faults during
@@ -72,7 +76,11 @@ typedef enum gas_status {
  *               array_len % 4 == 0 selects 128-bit vector loads/stores).
  *   num_arrays  N >= 0. array_len n >= 0. N == 0 or n <= 1: no-op, d_data may be NULL.
  *   n > gas_max_array_len(): GAS_ERROR_UNSUPPORTED, nothing enqueued.
- * One kernel launch per call.
+ * One kernel launch per call, except 512 < n <= 1024 with N >= 16384
+ * (BASELINE.json configs[1]-[4]): four launches, a device-routed pipeline
+ * (a sampler kernel picks, on the device, which of three kernels sorts the
+ * batch: value buckets, counting sort or sorting network; see
+ * csrc/sort1024.cuh) and its workspace (above).
  */
 GAS_API gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len, cudaStream_t stream);
 
@@ -90,9 +98,9 @@ GAS_API gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t ar
  *                  on the device first (with a stream synchronisation) and a
  *                  violation returns GAS_ERROR_INVALID_VALUE with nothing sorted.
  *   max_array_len > gas_max_array_len(): GAS_ERROR_UNSUPPORTED.
- * Workspace: 72 bytes of device memory per (device, stream) for dynamic
- * scheduling when max_array_len > 256, allocated on the first such call and
- * kept (re-zeroed in stream order by every call).
+ * Workspace: 72 bytes per call for dynamic scheduling when max_array_len >
+ * 256 (stream-ordered, from the library's pool; each call and each captured
+ * graph has its own).
  * One kernel launch per size class up to max_array_len (at most 17 launches:
  * powers of two up to 2048, then (2048,3072], (3072,4096], (4096,6144],
  * (6144,8192], (8192,12288], (12288,16384]). The launches are forked over 8
@@ -100,7 +108,9 @@ GAS_API gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t ar
  * use, with their fork/join events) and joined back into `stream` before the
  * call returns, so work enqueued later on `stream` still runs after the sort
  * and the call can be captured into a CUDA graph. GAS_OFFSETS_STREAMS=k
- * (1..8) sets the fan-out; 1 keeps every launch on `stream`.
+ * (1..8) sets the fan-out; 1 keeps every launch on `stream`. At most 64 caller
+ * streams per process get such a set; calls on further streams launch on
+ * `stream` alone. gas_release_stream() frees a stream's set.
  */
 GAS_API gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int64_t num_arrays,
                                    int32_t max_array_len, cudaStream_t stream);
@@ -130,6 +140,26 @@ GAS_API gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num
  * for later calls; concurrent host-path calls on one device are serialised.
  */
 GAS_API gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array_len);
+
+/*
+ * Host-memory variant of gas_sort_arrays_offsets (SURVEY.md §8(f) row f1 for
+ * ragged batches, the out-of-core spectra batches of P:L573-584): h_data and
+ * h_offsets are HOST memory (CSR as in gas_sort_arrays_offsets). The batch is
+ * cut at array boundaries into chunks of at most 128 MB (GAS_HOST_CHUNK_MB)
+ * and 2^20 arrays, streamed through the current device with the same
+ * overlapped H2D / sort / D2H as gas_sort_arrays_host, and written back in
+ * place. BLOCKING. Same argument rules as gas_sort_arrays_offsets; bytes
+ * outside [h_offsets[0], h_offsets[N]) are never read or written. Staging
+ * (data, pinned and device offsets buffers) is kept per device for later calls.
+ */
+GAS_API gas_status gas_sort_arrays_offsets_host(float* h_data, const int64_t* h_offsets, int64_t num_arrays,
+                                                int32_t max_array_len);
+
+/* Releases the side streams and events gas_sort_arrays_offsets created for
+   (current device, stream), after the work already enqueued on them has
+   finished (host-blocking on those streams only). Call it before destroying a
+   stream that was used with the offsets variant; a no-op for other streams. */
+GAS_API gas_status gas_release_stream(cudaStream_t stream);
 
 /* Largest supported array length of gas_sort_arrays / _offsets / _host: 16384,
    4x the paper's spectra bound of ~4000 peaks. */

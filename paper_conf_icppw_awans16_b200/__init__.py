@@ -10,6 +10,7 @@ or fails to load, every call raises.
     gas_sort_arrays_offsets(data, off) data: float32 CUDA [total], off: int64 CUDA [N+1]
     gas_sort_pairs(keys, vals)         stable key + uint32 payload (int32 tensor view)
     gas_sort_arrays_host(h)            h: [N, n] float32 CPU tensor (pinned for speed)
+    gas_sort_arrays_offsets_host(h, off) h: float32 CPU [total], off: int64 CPU [N+1]
 
 Order: IEEE 754-2008 totalOrder on the float32 bit patterns (C-1).
 """
@@ -49,6 +50,8 @@ def _load():
         lib.gas_sort_arrays_offsets.argtypes = [vp, vp, i64, i32, vp]
         lib.gas_sort_pairs.argtypes = [vp, vp, i64, i32, vp]
         lib.gas_sort_arrays_host.argtypes = [vp, i64, i32]
+        lib.gas_sort_arrays_offsets_host.argtypes = [vp, vp, i64, i32]
+        lib.gas_sort_arrays_offsets_host.restype = ctypes.c_int
         for f in (lib.gas_sort_arrays, lib.gas_sort_arrays_offsets, lib.gas_sort_pairs, lib.gas_sort_arrays_host):
             f.restype = ctypes.c_int
         lib.gas_max_array_len.restype = i32
@@ -56,6 +59,8 @@ def _load():
         lib.gas_status_string.restype = ctypes.c_char_p
         lib.gas_last_cuda_error.restype = ctypes.c_int
         lib.gas_launch_count.restype = i64
+        lib.gas_release_stream.argtypes = [vp]
+        lib.gas_release_stream.restype = ctypes.c_int
         _lib = lib
     return _lib
 
@@ -70,10 +75,20 @@ def _check(status: int, where: str):
         raise GasError(status, where)
 
 
-def _stream_ptr(stream) -> int:
+def _stream_ptr(stream, device) -> int:
+    """The stream to launch on: the caller's, or the current stream of the
+    tensor's device (never another device's stream)."""
     import torch
-    s = torch.cuda.current_stream() if stream is None else stream
+    s = torch.cuda.current_stream(device) if stream is None else stream
+    if s.device != device:
+        raise ValueError(f"stream is on {s.device}, data on {device}")
     return int(s.cuda_stream)
+
+
+def _same_device(where, a, *others):
+    for o in others:
+        if o.device != a.device:
+            raise ValueError(f"{where}: tensors on {a.device} and {o.device}")
 
 
 def _require_cuda(t, dtype_names, where):
@@ -94,14 +109,23 @@ def launch_count() -> int:
     return int(_load().gas_launch_count())
 
 
+def release_stream(stream) -> None:
+    """Free the side streams the offsets variant keeps for `stream` (a torch
+    stream or a raw cudaStream_t); call before destroying that stream."""
+    ptr = int(stream.cuda_stream) if hasattr(stream, "cuda_stream") else int(stream)
+    _check(_load().gas_release_stream(ptr or None), "gas_release_stream")
+
+
 def gas_sort_arrays(x, stream=None):
     """Sort every row of a [N, n] float32 CUDA tensor ascending, in place."""
     _require_cuda(x, ("float32",), "gas_sort_arrays")
     if x.dim() != 2:
         raise ValueError("gas_sort_arrays: expected [N, n]")
     N, n = x.shape
-    _check(_load().gas_sort_arrays(x.data_ptr() if x.numel() else None, N, n, _stream_ptr(stream)),
-           "gas_sort_arrays")
+    import torch
+    with torch.cuda.device(x.device):  # libgas launches on the current device
+        _check(_load().gas_sort_arrays(x.data_ptr() if x.numel() else None, N, n, _stream_ptr(stream, x.device)),
+               "gas_sort_arrays")
     return x
 
 
@@ -114,11 +138,15 @@ def gas_sort_arrays_offsets(data, offsets, max_array_len: int = 0, stream=None):
     """Sort data[offsets[i]:offsets[i+1]] for every i, in place."""
     _require_cuda(data, ("float32",), "gas_sort_arrays_offsets")
     _require_cuda(offsets, ("int64",), "gas_sort_arrays_offsets")
+    _same_device("gas_sort_arrays_offsets", data, offsets)
     N = offsets.numel() - 1
     if N < 0:
         raise ValueError("offsets must have N+1 >= 1 entries")
-    _check(_load().gas_sort_arrays_offsets(data.data_ptr() if data.numel() else None, offsets.data_ptr(), N,
-                                           max_array_len, _stream_ptr(stream)), "gas_sort_arrays_offsets")
+    import torch
+    with torch.cuda.device(data.device):
+        _check(_load().gas_sort_arrays_offsets(data.data_ptr() if data.numel() else None, offsets.data_ptr(), N,
+                                               max_array_len, _stream_ptr(stream, data.device)),
+               "gas_sort_arrays_offsets")
     return data
 
 
@@ -128,10 +156,14 @@ def gas_sort_pairs(keys, values, stream=None):
     _require_cuda(values, ("int32", "uint32", "float32"), "gas_sort_pairs")
     if keys.shape != values.shape or keys.dim() != 2:
         raise ValueError("gas_sort_pairs: keys and values must both be [N, n]")
+    _same_device("gas_sort_pairs", keys, values)
     N, n = keys.shape
-    _check(_load().gas_sort_pairs(keys.data_ptr() if keys.numel() else None,
-                                  values.data_ptr() if values.numel() else None, N, n, _stream_ptr(stream)),
-           "gas_sort_pairs")
+    import torch
+    with torch.cuda.device(keys.device):
+        _check(_load().gas_sort_pairs(keys.data_ptr() if keys.numel() else None,
+                                      values.data_ptr() if values.numel() else None, N, n,
+                                      _stream_ptr(stream, keys.device)),
+               "gas_sort_pairs")
     return keys, values
 
 
@@ -145,3 +177,20 @@ def gas_sort_arrays_host(h):
     N, n = h.shape
     _check(_load().gas_sort_arrays_host(h.data_ptr() if h.numel() else None, N, n), "gas_sort_arrays_host")
     return h
+
+
+def gas_sort_arrays_offsets_host(h, offsets, max_array_len: int = 0):
+    """Blocking sort of a ragged HOST batch (CSR offsets in host memory) through the GPU."""
+    import torch
+    for t, dt, name in ((h, torch.float32, "data"), (offsets, torch.int64, "offsets")):
+        if not isinstance(t, torch.Tensor) or t.is_cuda or t.dtype != dt or not t.is_contiguous():
+            raise TypeError(f"gas_sort_arrays_offsets_host: {name} must be a contiguous {dt} CPU tensor")
+    N = offsets.numel() - 1
+    if N < 0:
+        raise ValueError("offsets must have N+1 >= 1 entries")
+    _check(_load().gas_sort_arrays_offsets_host(h.data_ptr() if h.numel() else None, offsets.data_ptr(), N,
+                                                max_array_len), "gas_sort_arrays_offsets_host")
+    return h
+
+
+from . import dist, shard  # noqa: E402  (multi-GPU entry points; torch is imported lazily)

@@ -58,12 +58,35 @@ struct HostStaging {
       if (!buf[s]) e = cudaMalloc(&buf[s], bytes);
     return e;
   }
+  // offsets staging of gas_sort_arrays_offsets_host: pinned host + device, per slot
+  int64_t* off_h[kHostSlots] = {};
+  int64_t* off_d[kHostSlots] = {};
+  int64_t off_cap = 0;  // entries
+  cudaError_t ensure_offsets(int slots, int64_t entries) {
+    cudaError_t e = cudaSuccess;
+    if (entries > off_cap) {
+      for (int s = 0; s < kHostSlots; ++s) {
+        if (off_h[s]) { cudaFreeHost(off_h[s]); off_h[s] = nullptr; }
+        if (off_d[s]) { cudaFree(off_d[s]); off_d[s] = nullptr; }
+      }
+      off_cap = entries;
+    }
+    for (int s = 0; s < slots && e == cudaSuccess; ++s) {
+      if (!off_h[s]) e = cudaMallocHost(&off_h[s], off_cap * sizeof(int64_t));
+      if (e == cudaSuccess && !off_d[s]) e = cudaMalloc(&off_d[s], off_cap * sizeof(int64_t));
+    }
+    return e;
+  }
 };
 HostStaging g_staging[kMaxDevices];
 
 // Per-(device, caller stream) side streams of the offsets variant: the class
-// launches fork over them and join back (see gas_sort_arrays_offsets).
+// launches fork over them and join back (see gas_sort_arrays_offsets). At most
+// kMaxSideSets caller streams get a set (8 streams + 9 events each); calls on
+// further streams launch every class on the caller's stream.
+// gas_release_stream() destroys a stream's set.
 constexpr int kMaxSide = 8;
+constexpr size_t kMaxSideSets = 64;
 struct SideStreams {
   cudaStream_t s[kMaxSide];
   cudaEvent_t fork, join[kMaxSide];
@@ -81,44 +104,49 @@ int offsets_streams() {
   return k;
 }
 
+void destroy_side(SideStreams* ss) {
+  for (int i = 0; i < kMaxSide; ++i) {
+    if (ss->s[i]) cudaStreamDestroy(ss->s[i]);
+    if (ss->join[i]) cudaEventDestroy(ss->join[i]);
+  }
+  if (ss->fork) cudaEventDestroy(ss->fork);
+  delete ss;
+}
+
+// *out = nullptr (and success) when the cache is full: the caller then uses one stream.
 cudaError_t side_streams_for(cudaStream_t stream, SideStreams** out) {
+  *out = nullptr;
   int dev = 0;
   cudaError_t e = cudaGetDevice(&dev);
   if (e != cudaSuccess) return e;
   std::lock_guard<std::mutex> lock(g_side_mu);
-  auto& slot = g_side[{dev, stream}];
-  if (!slot) {
-    SideStreams* ss = new SideStreams();
-    e = cudaEventCreateWithFlags(&ss->fork, cudaEventDisableTiming);
-    for (int i = 0; i < kMaxSide && e == cudaSuccess; ++i) {
-      e = cudaStreamCreateWithFlags(&ss->s[i], cudaStreamNonBlocking);
-      if (e == cudaSuccess) e = cudaEventCreateWithFlags(&ss->join[i], cudaEventDisableTiming);
-    }
-    if (e != cudaSuccess) return e;  // (leaks the partial set; only on a failing device)
-    slot = ss;
+  auto it = g_side.find({dev, stream});
+  if (it != g_side.end()) {
+    *out = it->second;
+    return cudaSuccess;
   }
-  *out = slot;
+  if (g_side.size() >= kMaxSideSets) return cudaSuccess;
+  SideStreams* ss = new SideStreams();
+  for (int i = 0; i < kMaxSide; ++i) { ss->s[i] = nullptr; ss->join[i] = nullptr; }
+  ss->fork = nullptr;
+  e = cudaEventCreateWithFlags(&ss->fork, cudaEventDisableTiming);
+  for (int i = 0; i < kMaxSide && e == cudaSuccess; ++i) {
+    e = cudaStreamCreateWithFlags(&ss->s[i], cudaStreamNonBlocking);
+    if (e == cudaSuccess) e = cudaEventCreateWithFlags(&ss->join[i], cudaEventDisableTiming);
+  }
+  if (e != cudaSuccess) {
+    destroy_side(ss);
+    return e;
+  }
+  g_side[{dev, stream}] = ss;
+  *out = ss;
   return cudaSuccess;
 }
 
-// Per-(device, stream) window counters of the offsets variant (see there).
+// Window counters of the offsets variant's dynamic scheduling: 9 x 8 bytes
+// per call, stream-ordered from the library's memory pool (each call and each
+// captured graph owns its counters: concurrent calls never share them).
 constexpr int kCounters = 9;
-std::mutex g_ctr_mu;
-std::map<std::pair<int, cudaStream_t>, unsigned long long*> g_ctr;
-
-cudaError_t counters_for(cudaStream_t stream, unsigned long long** out) {
-  int dev = 0;
-  cudaError_t e = cudaGetDevice(&dev);
-  if (e != cudaSuccess) return e;
-  std::lock_guard<std::mutex> lock(g_ctr_mu);
-  auto& slot = g_ctr[{dev, stream}];
-  if (!slot) {
-    e = cudaMalloc(&slot, kCounters * sizeof(unsigned long long));
-    if (e != cudaSuccess) { slot = nullptr; return e; }
-  }
-  *out = slot;
-  return cudaSuccess;
-}
 
 bool env_check() {
   const char* v = std::getenv("GAS_CHECK");
@@ -167,15 +195,23 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
     if (h) return GAS_ERROR_INVALID_VALUE;
   }
   uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
-  // 9 window counters for the bucket classes' dynamic scheduling: 72 bytes per
-  // (device, stream), allocated on first use and re-zeroed in stream order by
-  // every call (calls on one stream are ordered; different streams never share)
+  // 9 window counters for the bucket classes' dynamic scheduling (72 bytes per call)
   unsigned long long* ctr = nullptr;
   if (max_array_len > 256) {
-    cudaError_t e = counters_for(stream, &ctr);
-    if (e == cudaSuccess) e = cudaMemsetAsync(ctr, 0, kCounters * sizeof(unsigned long long), stream);
+    void* p = nullptr;
+    cudaError_t e = ws_alloc(&p, kCounters * sizeof(unsigned long long), stream);
+    if (e == cudaSuccess) e = cudaMemsetAsync(p, 0, kCounters * sizeof(unsigned long long), stream);
     if (e != cudaSuccess) return cuda_fail(e);
+    ctr = static_cast<unsigned long long*>(p);
   }
+  // every exit below frees the counters on `stream`, after the work that uses them
+  auto release = [&](cudaError_t e) -> gas_status {
+    if (ctr) {
+      const cudaError_t f = cudaFreeAsync(ctr, stream);
+      if (e == cudaSuccess) e = f;
+    }
+    return e == cudaSuccess ? GAS_SUCCESS : cuda_fail(e);
+  };
   // size classes: 2, 4, ..., 2048 (len in (P/2, P]), then (2048, 3072] and (3072, 4096]
   const int32_t classes[] = {2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288, 16384};
   const int32_t lower[] = {1, 2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288};
@@ -189,15 +225,15 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
   SideStreams* ss = nullptr;
   if (offsets_streams() > 1 && nclass > 1) {
     const cudaError_t e = side_streams_for(stream, &ss);
-    if (e != cudaSuccess) return cuda_fail(e);
+    if (e != cudaSuccess) return release(e);
   }
   if (!ss) {
     for (int c = 0; c < nclass; ++c) {
       const cudaError_t e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, ctr, stream);
-      if (e != cudaSuccess) return cuda_fail(e);
+      if (e != cudaSuccess) return release(e);
       launch_counter() += 1;
     }
-    return GAS_SUCCESS;
+    return release(cudaSuccess);
   }
   std::lock_guard<std::mutex> lock(ss->mu);
   const int K = offsets_streams();
@@ -213,7 +249,7 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
     const cudaError_t w = r == cudaSuccess ? cudaStreamWaitEvent(stream, ss->join[i], 0) : r;
     if (e == cudaSuccess) e = w;
   }
-  return e == cudaSuccess ? GAS_SUCCESS : cuda_fail(e);
+  return release(e);
 }
 
 gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays, int32_t array_len,
@@ -273,6 +309,82 @@ gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array
   }
   if (status != GAS_SUCCESS) return status;
   if (e != cudaSuccess) return cuda_fail(e);
+  return GAS_SUCCESS;
+}
+
+gas_status gas_sort_arrays_offsets_host(float* h_data, const int64_t* h_offsets, int64_t num_arrays,
+                                        int32_t max_array_len) {
+  if (num_arrays < 0 || max_array_len < 0) return GAS_ERROR_INVALID_VALUE;
+  if (max_array_len == 0) max_array_len = kMaxLen;
+  if (max_array_len > kMaxLen) return GAS_ERROR_UNSUPPORTED;
+  if (num_arrays == 0 || max_array_len <= 1) return GAS_SUCCESS;
+  if (h_offsets == nullptr || h_data == nullptr || (reinterpret_cast<uintptr_t>(h_data) & 3u))
+    return GAS_ERROR_INVALID_VALUE;
+  const char* env_chunk = std::getenv("GAS_HOST_CHUNK_MB");
+  const char* env_slots = std::getenv("GAS_HOST_SLOTS");
+  const int64_t chunk_elems = ((env_chunk ? std::atoll(env_chunk) : 128ll) << 20) / 4;
+  const int64_t max_chunk_arrays = 1 << 20;  // bounds the offsets staging (8 MB per slot)
+  int slots = env_slots ? std::atoi(env_slots) : 3;
+  slots = slots < 1 ? 1 : (slots > kHostSlots ? kHostSlots : slots);
+  int dev = 0;
+  cudaError_t e = cudaGetDevice(&dev);
+  if (e != cudaSuccess) return cuda_fail(e);
+  if (dev < 0 || dev >= kMaxDevices) return GAS_ERROR_UNSUPPORTED;
+  HostStaging& hs = g_staging[dev];
+  std::lock_guard<std::mutex> lock(hs.mu);
+  const int64_t per = chunk_elems > max_array_len ? chunk_elems : max_array_len;
+  e = hs.ensure(slots, per * 4);
+  if (e == cudaSuccess) e = hs.ensure_offsets(slots, max_chunk_arrays + 1);
+  if (e != cudaSuccess) return cuda_fail(e);
+  gas_status status = GAS_SUCCESS;
+  int64_t a = 0;
+  for (int64_t c = 0; a < num_arrays && e == cudaSuccess && status == GAS_SUCCESS; ++c) {
+    // chunk = arrays [a, b): whole arrays, at most `per` elements and max_chunk_arrays arrays
+    int64_t b = a + 1;
+    while (b < num_arrays && b - a < max_chunk_arrays && h_offsets[b + 1] - h_offsets[a] <= per) ++b;
+    const int sl = (int)(c % slots);
+    e = cudaStreamSynchronize(hs.st[sl]);  // the slot's previous chunk is done with its staging
+    if (e != cudaSuccess) break;
+    const int64_t base = h_offsets[a], elems = h_offsets[b] - base;
+    if (elems < 0 || elems > per) { status = GAS_ERROR_INVALID_VALUE; break; }
+    std::memcpy(hs.off_h[sl], h_offsets + a, (b - a + 1) * sizeof(int64_t));
+    e = cudaMemcpyAsync(hs.off_d[sl], hs.off_h[sl], (b - a + 1) * sizeof(int64_t), cudaMemcpyHostToDevice, hs.st[sl]);
+    if (e == cudaSuccess && elems > 0)
+      e = cudaMemcpyAsync(hs.buf[sl], h_data + base, elems * 4, cudaMemcpyHostToDevice, hs.st[sl]);
+    if (e != cudaSuccess) break;
+    // the device offsets are the caller's (not rebased): the data pointer is shifted instead
+    status = gas_sort_arrays_offsets(hs.buf[sl] - base, hs.off_d[sl], b - a, max_array_len, hs.st[sl]);
+    if (status != GAS_SUCCESS) break;
+    if (elems > 0) e = cudaMemcpyAsync(h_data + base, hs.buf[sl], elems * 4, cudaMemcpyDeviceToHost, hs.st[sl]);
+    a = b;
+  }
+  for (int sl = 0; sl < slots; ++sl) {
+    const cudaError_t e2 = cudaStreamSynchronize(hs.st[sl]);
+    if (e == cudaSuccess) e = e2;
+  }
+  if (status != GAS_SUCCESS) return status;
+  if (e != cudaSuccess) return cuda_fail(e);
+  return GAS_SUCCESS;
+}
+
+gas_status gas_release_stream(cudaStream_t stream) {
+  int dev = 0;
+  const cudaError_t e = cudaGetDevice(&dev);
+  if (e != cudaSuccess) return cuda_fail(e);
+  SideStreams* ss = nullptr;
+  {
+    std::lock_guard<std::mutex> lock(g_side_mu);
+    auto it = g_side.find({dev, stream});
+    if (it == g_side.end()) return GAS_SUCCESS;
+    ss = it->second;
+    g_side.erase(it);
+  }
+  {
+    std::lock_guard<std::mutex> lock(ss->mu);  // a call still enqueueing on this set finishes first
+  }
+  for (int i = 0; i < kMaxSide; ++i)
+    if (ss->s[i]) cudaStreamSynchronize(ss->s[i]);
+  destroy_side(ss);
   return GAS_SUCCESS;
 }
 

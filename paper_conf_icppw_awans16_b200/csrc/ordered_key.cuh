@@ -5,7 +5,8 @@
 //     key(u) = u ^ (sign(u) ? 0xFFFFFFFF : 0x80000000)
 // (negatives: all bits flipped, so larger magnitude -> smaller key and
 //  -NaN < -inf; positives: sign bit set, so every positive > every negative).
-// Checked over all 2^32 patterns in tests/test_ordered_key.py.
+// Checked over all 2^32 patterns, through the sort kernels, by
+// tests/test_ordered_key.py::test_every_bit_pattern_through_the_gpu.
 //
 // Sorting happens on keys only; the kernels never apply float arithmetic to
 // data (no NaN quieting, no FTZ), so the output is a permutation of the input

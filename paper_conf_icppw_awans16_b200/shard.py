@@ -56,21 +56,29 @@ def max_over_ranks(value: float, device=None) -> float:
 
 
 def gather_to_rank0(local, counts: Sequence[int], dst: int = 0):
-    """Optional gather of variable-size sorted shards to rank `dst` (point to
-    point send/recv; NCCL over NVLink on B200). Returns the concatenation on
-    `dst`, None elsewhere. Not on the timed path."""
+    """Optional gather of variable-size sorted shards to rank `dst`: the
+    receiver preallocates the whole result and posts every receive into its
+    slice at once (one batch of point-to-point ops: an NCCL group over NVLink
+    on B200), the senders post one send each. Returns the result on `dst`,
+    None elsewhere. Not on the timed path."""
     import torch
     import torch.distributed as dist
     rank, world = dist.get_rank(), dist.get_world_size()
     if rank != dst:
-        dist.send(local.contiguous(), dst)
+        if local.shape[0]:
+            for req in dist.batch_isend_irecv([dist.P2POp(dist.isend, local.contiguous(), dst)]):
+                req.wait()
         return None
-    parts = []
+    out = torch.empty((sum(counts),) + tuple(local.shape[1:]), dtype=local.dtype, device=local.device)
+    ops, start = [], 0
     for r in range(world):
+        part = out[start:start + counts[r]]
         if r == rank:
-            parts.append(local)
-        else:
-            buf = torch.empty((counts[r],) + tuple(local.shape[1:]), dtype=local.dtype, device=local.device)
-            dist.recv(buf, r)
-            parts.append(buf)
-    return torch.cat(parts)
+            part.copy_(local)
+        elif counts[r]:
+            ops.append(dist.P2POp(dist.irecv, part, r))
+        start += counts[r]
+    if ops:
+        for req in dist.batch_isend_irecv(ops):
+            req.wait()
+    return out

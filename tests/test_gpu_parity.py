@@ -383,3 +383,104 @@ def test_cuda_graph_capture_and_replay():
     expect = rdata.copy()
     oracle.sort_arrays_offsets_(expect, off)
     np.testing.assert_array_equal(to_host(r), expect)
+
+
+def _offsets_batch(N=3000, seed=77):
+    lens = datagen.lengths(seed, 0, N, 100, 4000)
+    off = datagen.offsets_from_lengths(lens)
+    host = datagen.ragged("spectra_intensity", seed, 0, off)
+    return host, off
+
+
+def test_offsets_first_call_on_fresh_stream_does_not_synchronise():
+    """The offsets variant's workspace is stream-ordered (no cudaMalloc): a call
+    on a brand-new stream returns while another stream is still busy."""
+    host, off = _offsets_batch()
+    d, o = to_dev(host), torch.from_numpy(off).to(DEV)
+    busy = torch.cuda.Stream()
+    fresh = torch.cuda.Stream()
+    with torch.cuda.stream(busy):
+        torch.cuda._sleep(2_000_000_000)  # ~1 s of spinning on `busy`
+        done = torch.cuda.Event()
+        done.record(busy)
+    gas.gas_sort_arrays_offsets(d.view(torch.float32), o, 4000, stream=fresh)
+    assert not done.query(), "the call waited for unrelated work (device synchronisation)"
+    torch.cuda.synchronize()
+    want = host.copy()
+    oracle.sort_arrays_offsets_(want, off)
+    np.testing.assert_array_equal(to_host(d), want)
+    gas.release_stream(fresh)
+
+
+def test_offsets_two_threads_one_stream():
+    """Two host threads sorting different batches on the same stream: each
+    call has its own window counters, so neither skips arrays."""
+    import threading
+    s = torch.cuda.Stream()
+    batches = [_offsets_batch(2500, seed) for seed in (101, 202)]
+    devs = [(to_dev(h), torch.from_numpy(o).to(DEV)) for h, o in batches]
+    errors = []
+
+    def work(i):
+        try:
+            for _ in range(20):
+                gas.gas_sort_arrays_offsets(devs[i][0].view(torch.float32), devs[i][1], 4000, stream=s)
+        except Exception as e:  # pragma: no cover
+            errors.append(e)
+
+    ts = [threading.Thread(target=work, args=(i,)) for i in range(2)]
+    [t.start() for t in ts]
+    [t.join() for t in ts]
+    torch.cuda.synchronize()
+    assert not errors
+    for (h, o), (d, _) in zip(batches, devs):
+        want = h.copy()
+        oracle.sort_arrays_offsets_(want, o)
+        np.testing.assert_array_equal(to_host(d), want)
+    gas.release_stream(s)
+
+
+def test_release_stream_then_reuse():
+    host, off = _offsets_batch(500, 9)
+    s = torch.cuda.Stream()
+    for _ in range(2):
+        d, o = to_dev(host), torch.from_numpy(off).to(DEV)
+        gas.gas_sort_arrays_offsets(d.view(torch.float32), o, 4000, stream=s)
+        torch.cuda.synchronize()
+        gas.release_stream(s)
+        want = host.copy()
+        oracle.sort_arrays_offsets_(want, off)
+        np.testing.assert_array_equal(to_host(d), want)
+    gas.release_stream(torch.cuda.Stream())  # never used: a no-op
+
+
+def test_tensor_on_other_device_is_rejected_or_handled():
+    """The wrappers launch on the tensor's own device and stream."""
+    x = to_dev(datagen.fixed("paper_uniform", 5, 0, 50, 1000)).view(torch.float32).view(50, 1000)
+    gas.gas_sort_arrays(x)
+    other = torch.cuda.Stream()
+    gas.gas_sort_arrays(x, stream=other)
+    torch.cuda.synchronize()
+    with pytest.raises((TypeError, ValueError)):  # offsets on the host, data on the GPU
+        gas.gas_sort_arrays_offsets(x.view(-1), torch.zeros(2, dtype=torch.int64), 0)
+
+
+@pytest.mark.parametrize("chunk_mb", [None, "1"])
+def test_offsets_host_entry_point(monkeypatch, chunk_mb):
+    """gas_sort_arrays_offsets_host: ragged batch in host memory, chunked at array
+    boundaries (1 MB chunks force many chunks and slot reuse); empty arrays and
+    a gap before the first array; bit-exact; bytes outside the batch untouched."""
+    if chunk_mb:
+        monkeypatch.setenv("GAS_HOST_CHUNK_MB", chunk_mb)
+    lens = datagen.lengths(31, 0, 4000, 0, 4000)
+    lens[::97] = 0
+    off = datagen.offsets_from_lengths(lens) + 5  # the batch starts 5 floats into the buffer
+    body = datagen.ragged("special_mix", 31, 0, off - 5)
+    buf = np.concatenate([np.full(5, CANARY, np.uint32), body, np.full(3, CANARY, np.uint32)])
+    h = torch.from_numpy(buf.copy().view(np.float32)).pin_memory()
+    gas.gas_sort_arrays_offsets_host(h, torch.from_numpy(off), 4000)
+    got = h.numpy().view(np.uint32)
+    want = body.copy()
+    oracle.sort_arrays_offsets_(want, off - 5)
+    np.testing.assert_array_equal(got[5:-3], want)
+    assert np.all(got[:5] == CANARY) and np.all(got[-3:] == CANARY)
