@@ -15,7 +15,8 @@
 namespace {
 
 constexpr int32_t kMaxPairsLen = 8192;  // 64-bit network elements: 8 KB of SMEM per 1024
-constexpr int32_t kMaxLen = 16384;  // 4x the spectra bound of P:L170-173
+constexpr int32_t kMaxLen = 65536;       // fixed-length arrays: 16x the spectra bound of P:L170-173
+constexpr int32_t kMaxOffsetsLen = 16384;  // variable-length classes (one CTA per array)
 
 thread_local int g_last_cuda_error = 0;
 
@@ -164,19 +165,20 @@ gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len,
   if (d_data == nullptr || (reinterpret_cast<uintptr_t>(d_data) & 3u)) return GAS_ERROR_INVALID_VALUE;
   uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
   const bool vec = (reinterpret_cast<uintptr_t>(d_data) & 15u) == 0 && (array_len & 3) == 0;
-  const cudaError_t e = array_len <= 512    ? dispatch_fixed_small(vec, d, num_arrays, array_len, stream)
-                        : array_len <= 1024 ? dispatch_fixed_1024(vec, d, num_arrays, array_len, stream)
-                                            : dispatch_fixed_cta(vec, d, num_arrays, array_len, stream);
+  const cudaError_t e = array_len <= 512     ? dispatch_fixed_small(vec, d, num_arrays, array_len, stream)
+                        : array_len <= 1024  ? dispatch_fixed_1024(vec, d, num_arrays, array_len, stream)
+                        : array_len <= 16384 ? dispatch_fixed_cta(vec, d, num_arrays, array_len, stream)
+                                             : dispatch_fixed_cluster(vec, d, num_arrays, array_len, stream);
   if (e != cudaSuccess) return cuda_fail(e);
-  if (array_len <= 512 || array_len > 1024) launch_counter() += 1;  // the 1024 class counts its own launches
+  if (array_len <= 512 || (array_len > 1024 && array_len <= 16384)) launch_counter() += 1;  // others count their own
   return GAS_SUCCESS;
 }
 
 gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int64_t num_arrays,
                                    int32_t max_array_len, cudaStream_t stream) {
   if (num_arrays < 0 || max_array_len < 0) return GAS_ERROR_INVALID_VALUE;
-  if (max_array_len == 0) max_array_len = kMaxLen;
-  if (max_array_len > kMaxLen) return GAS_ERROR_UNSUPPORTED;
+  if (max_array_len == 0) max_array_len = kMaxOffsetsLen;
+  if (max_array_len > kMaxOffsetsLen) return GAS_ERROR_UNSUPPORTED;
   if (num_arrays == 0 || max_array_len <= 1) return GAS_SUCCESS;
   if (d_offsets == nullptr || (reinterpret_cast<uintptr_t>(d_offsets) & 7u)) return GAS_ERROR_INVALID_VALUE;
   if (d_data == nullptr || (reinterpret_cast<uintptr_t>(d_data) & 3u)) return GAS_ERROR_INVALID_VALUE;
@@ -315,8 +317,8 @@ gas_status gas_sort_arrays_host(float* h_data, int64_t num_arrays, int32_t array
 gas_status gas_sort_arrays_offsets_host(float* h_data, const int64_t* h_offsets, int64_t num_arrays,
                                         int32_t max_array_len) {
   if (num_arrays < 0 || max_array_len < 0) return GAS_ERROR_INVALID_VALUE;
-  if (max_array_len == 0) max_array_len = kMaxLen;
-  if (max_array_len > kMaxLen) return GAS_ERROR_UNSUPPORTED;
+  if (max_array_len == 0) max_array_len = kMaxOffsetsLen;
+  if (max_array_len > kMaxOffsetsLen) return GAS_ERROR_UNSUPPORTED;
   if (num_arrays == 0 || max_array_len <= 1) return GAS_SUCCESS;
   if (h_offsets == nullptr || h_data == nullptr || (reinterpret_cast<uintptr_t>(h_data) & 3u))
     return GAS_ERROR_INVALID_VALUE;

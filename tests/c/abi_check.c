@@ -16,13 +16,14 @@ static int fails = 0;
 static uint32_t key(uint32_t u) { return u ^ ((u >> 31) ? 0xFFFFFFFFu : 0x80000000u); }
 
 int main(int argc, char** argv) {
-  CHECK(gas_max_array_len() == 16384);
+  CHECK(gas_max_array_len() == 65536);
   CHECK(strcmp(gas_status_string(GAS_SUCCESS), "GAS_SUCCESS") == 0);
   CHECK(gas_sort_arrays(NULL, 0, 1000, 0) == GAS_SUCCESS);
   CHECK(gas_sort_arrays(NULL, 5, 1, 0) == GAS_SUCCESS);
   CHECK(gas_sort_arrays(NULL, -1, 10, 0) == GAS_ERROR_INVALID_VALUE);
   CHECK(gas_sort_arrays(NULL, 10, 10, 0) == GAS_ERROR_INVALID_VALUE);
-  CHECK(gas_sort_arrays((float*)(uintptr_t)0x1000, 10, 16385, 0) == GAS_ERROR_UNSUPPORTED);
+  CHECK(gas_sort_arrays((float*)(uintptr_t)0x1000, 10, 65537, 0) == GAS_ERROR_UNSUPPORTED);
+  CHECK(gas_sort_arrays_offsets((float*)(uintptr_t)0x1000, (const int64_t*)(uintptr_t)0x2000, 10, 16385, 0) == GAS_ERROR_UNSUPPORTED);
   CHECK(gas_sort_pairs((float*)(uintptr_t)0x1000, (uint32_t*)(uintptr_t)0x2000, 10, 8193, 0) == GAS_ERROR_UNSUPPORTED);
   CHECK(gas_sort_arrays_offsets(NULL, NULL, 0, 0, 0) == GAS_SUCCESS);
   CHECK(gas_sort_arrays_host(NULL, 3, 10) == GAS_ERROR_INVALID_VALUE);

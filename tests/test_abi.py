@@ -44,7 +44,7 @@ def test_status_strings_and_limits():
     assert lib.gas_status_string(1) == b"GAS_ERROR_INVALID_VALUE"
     assert lib.gas_status_string(2) == b"GAS_ERROR_UNSUPPORTED"
     assert lib.gas_status_string(3) == b"GAS_ERROR_CUDA"
-    assert gas.max_array_len() == 16384
+    assert gas.max_array_len() == 65536
     assert lib.gas_last_cuda_error() == 0
 
 
@@ -61,7 +61,8 @@ def test_argument_validation_without_launch():
     assert lib.gas_sort_arrays(None, 10, 10, None) == 1
     assert lib.gas_sort_arrays(ctypes.c_void_p(0x1002), 10, 10, None) == 1  # not 4-byte aligned
     # unsupported length
-    assert lib.gas_sort_arrays(ctypes.c_void_p(0x1000), 10, 16385, None) == 2
+    assert lib.gas_sort_arrays(ctypes.c_void_p(0x1000), 10, 65537, None) == 2
+    assert lib.gas_sort_arrays_offsets(ctypes.c_void_p(0x1000), ctypes.c_void_p(0x2000), 10, 16385, None) == 2
     assert lib.gas_sort_pairs(ctypes.c_void_p(0x1000), ctypes.c_void_p(0x2000), 10, 8193, None) == 2
     assert lib.gas_sort_arrays_offsets(ctypes.c_void_p(0x1000), ctypes.c_void_p(0x2000), 10, 20000, None) == 2
     assert lib.gas_sort_arrays_offsets(None, None, 0, 0, None) == 0
@@ -69,7 +70,7 @@ def test_argument_validation_without_launch():
     assert lib.gas_sort_arrays_offsets(ctypes.c_void_p(0x1000), ctypes.c_void_p(0x2004), 5, 0, None) == 1
     assert lib.gas_sort_arrays_host(None, 0, 10) == 0
     assert lib.gas_sort_arrays_host(None, 3, 10) == 1
-    assert lib.gas_sort_arrays_host(ctypes.c_void_p(0x1000), 3, 20000) == 2
+    assert lib.gas_sort_arrays_host(ctypes.c_void_p(0x1000), 3, 70000) == 2
     assert lib.gas_launch_count() == before
 
 
