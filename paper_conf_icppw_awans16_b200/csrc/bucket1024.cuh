@@ -60,6 +60,9 @@ namespace gas {
 #ifndef GAS_BK_GROUP  // keys whose atomics are issued back to back before their scatter stores
 #define GAS_BK_GROUP 4
 #endif
+#ifndef GAS_BK_TMA_STORE  // 1: the staged sorted array leaves through one TMA bulk store (cp.async.bulk) instead of 8 LDS.128 + STG.128 per lane
+#define GAS_BK_TMA_STORE 1
+#endif
 #ifndef GAS_BK_PREFETCH  // L2 prefetch of the array this warp sorts GAS_BK_PREFETCH iterations ahead (0 = off)
 #define GAS_BK_PREFETCH 1
 #endif
@@ -334,6 +337,10 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + (a + GAS_BK_PREFETCH * nwarps) * (int64_t)n),
                    "r"((uint32_t)n * 4u) : "memory");
 #endif
+#if GAS_BK_TMA_STORE
+    if (lane == 0) asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory");  // the previous bulk store has read the staging
+    __syncwarp();
+#endif
     // slots past the end repeat k[0] so that min / max need no predicates
 #pragma unroll
     for (int q = 4; q < 8; ++q) {
@@ -445,6 +452,17 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 #pragma unroll
         for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
       }
+#if GAS_BK_TMA_STORE
+      if (raw) {  // the staged array is contiguous: one TMA bulk store (the copy engine reads shared memory)
+        asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+        __syncwarp();
+        if (lane == 0) {
+          asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;"
+                       ::"l"(dst), "r"(stage_sa), "r"((uint32_t)n * 4u) : "memory");
+          asm volatile("cp.async.bulk.commit_group;" ::: "memory");
+        }
+      } else {
+#else
       __syncwarp();
       if (raw) {
 #pragma unroll
@@ -453,6 +471,8 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
           stg_cs_if(q < 4 || c < nc, dst + c, lds128(stage_sa + c * 16));
         }
       } else {
+#endif
+        __syncwarp();
 #pragma unroll
         for (int q = 0; q < 8; ++q) {
           const int c = lane + 32 * q;
@@ -467,6 +487,9 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     }
     __syncwarp();
   }
+#if GAS_BK_TMA_STORE
+  if (lane == 0) asm volatile("cp.async.bulk.wait_group 0;" ::: "memory");  // stores complete before the CTA exits
+#endif
 }
 
 // The same kernel for rows at any 4-byte alignment (n % 4 != 0 or an
