@@ -65,6 +65,9 @@ template <int WR> __host__ __device__ constexpr int bkc_min_blocks() { return bk
 #ifndef GAS_BKC_PREFETCH
 #define GAS_BKC_PREFETCH 1
 #endif
+#ifndef GAS_BKC_TMA_STORE  // output of the CTA bucket path through one TMA bulk store (see bucket_sort_cta)
+#define GAS_BKC_TMA_STORE 1
+#endif
 
 // Arrays per CTA: GROUPS independent thread groups of WR warps share one CTA
 // (one CTA per SM; GAS_BKC_GROUPS=0: one group per CTA, several CTAs per SM)
@@ -91,7 +94,14 @@ __device__ __forceinline__ void bar_cta(uint32_t bar) {
 // (0: the group is the whole CTA).
 // RV: key slots r < RV are always inside the array (n > 32 WR RV; 16 for the
 // classes (P/2, P], 8 when the W = 1 kernel serves 256 < n <= 512).
-template <int W, int WR, bool VEC, int RV = 16>
+// TMA: the bucket path's output leaves through one TMA bulk store of the
+// staged array (thread 0 of the group issues it; the sorted key i is staged at
+// word i + head, head = the array's word offset inside its 16-byte chunk, so
+// that shared source and global destination share their alignment; the <= 3
+// words before the first and after the last 16-byte boundary are stored one by
+// one). Thread 0 waits for the previous store's reads before the group's first
+// row write of the next array; the kernel waits for completion before exiting.
+template <int W, int WR, bool VEC, int RV = 16, bool TMA = (GAS_BKC_TMA_STORE != 0)>
 __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int n, unsigned char* sm, uint32_t one,
                                                 int t, uint32_t bar) {
   using C = BkCta<W, WR>;
@@ -107,6 +117,8 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
   const uint32_t row0 = slot_sa + t * (kBkRowWords * 4);  // rows of buckets t and t + T
   const uint32_t row1 = row0 + T * (kBkRowWords * 4);
   const int nc = n >> 2;
+  const int head = TMA ? (int)((reinterpret_cast<uintptr_t>(arr) >> 2) & 3u) : 0;  // staging shift (0 when VEC)
+  if (TMA && t == 0) asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory");  // ordered by the first barrier
   // key r of this thread: VEC element 4 (t + T (r/4)) + r%4, else element t + T r
   auto valid = [&](int r) -> bool {
     if (VEC) return (r >> 2) < 4 || t + T * (r >> 2) < nc;
@@ -241,7 +253,7 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
     for (int rho = 0; rho < 2; ++rho) {
       const uint32_t tb = rho ? t0 : t1;
       const uint32_t row = rho ? row0 : row1;
-      const uint32_t ob = stage_sa + (rho ? base0 : base1) * 4;
+      const uint32_t ob = stage_sa + ((rho ? base0 : base1) + head) * 4;
       if (rho == 0) {
 #pragma unroll
         for (int i = 0; i < 32; ++i) k[i] = kPadKey;
@@ -252,9 +264,27 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
       // second round reads rows 0 .. T-1, which staging never touches)
       if (rho == 0) bar_cta<WR>(bar);
       sortn_bk<32>(k, one);
+      if (TMA && !raw) {  // the bulk store copies bits: stage transformed keys (k keeps the keys: the
+#pragma unroll            // second round uses them as padding)
+        for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, bits_from_key(k[i]));
+      } else {
 #pragma unroll
-      for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
+        for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
+      }
     }
+    if constexpr (TMA) {
+      asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // this thread's staging writes -> async proxy
+      bar_cta<WR>(bar);
+      const int h0 = (4 - head) & 3, h1 = h0 + ((n - h0) & ~3);  // [h0, h1): 16-byte aligned in both memories
+      if (t == 0 && h1 > h0) {
+        asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;"
+                     ::"l"(arr + h0), "r"(stage_sa + (uint32_t)(head + h0) * 4u), "r"((uint32_t)(h1 - h0) * 4u)
+                     : "memory");
+        asm volatile("cp.async.bulk.commit_group;" ::: "memory");
+      }
+      if (t < h0) st_stream(arr + t, lds32(stage_sa + (head + t) * 4));
+      else if (t >= 4 && t - 4 + h1 < n) st_stream(arr + (t - 4 + h1), lds32(stage_sa + (head + t - 4 + h1) * 4));
+    } else {
     bar_cta<WR>(bar);
     if constexpr (VEC) {
       uint4* dst = reinterpret_cast<uint4*>(arr);
@@ -280,6 +310,7 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
         }
       }
     }
+    }  // !TMA
   } else {
     // ---- fallback: the whole-array network (warp1024.cuh sort_cta)
 #pragma unroll
@@ -327,6 +358,7 @@ __global__ void __launch_bounds__(bkc_block<WR>(), bkc_launch_min_blocks<WR>())
 #endif
     bucket_sort_cta<W, WR, VEC>(d + a * (int64_t)n, n, sm, one, t, bar);
   }
+  if (GAS_BKC_TMA_STORE && t == 0) asm volatile("cp.async.bulk.wait_group 0;" ::: "memory");
 }
 
 // Variable length: the arrays with LO < len <= HI (P/2 <= LO, HI <= P), found
@@ -372,6 +404,7 @@ __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
       bucket_sort_cta<W, WR, false, RV>(d + lo, len, sm, one, t, bar);
     }
   }
+  if (GAS_BKC_TMA_STORE && t == 0) asm volatile("cp.async.bulk.wait_group 0;" ::: "memory");
 }
 
 }  // namespace gas

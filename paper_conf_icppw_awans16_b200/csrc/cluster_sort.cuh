@@ -51,6 +51,8 @@ __device__ __forceinline__ void cl_part_sort(uint32_t* arr, int len, unsigned ch
 // Parts of <= 256 keys: the first warp sorts them with the 1024-key network.
 __device__ __forceinline__ void cl_small_sort(uint32_t* arr, int len, unsigned char* sm, uint32_t one, int t) {
   if (t >= 32) return;
+  if (GAS_BKC_TMA_STORE && t == 0) asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory");  // sm is scratch here
+  __syncwarp();
   uint32_t k[32];
 #pragma unroll
   for (int r = 0; r < 32; ++r) {
@@ -206,6 +208,7 @@ __global__ void __cluster_dims__(kClC, 1, 1) __launch_bounds__(kClT, 1)
     if (plen <= kClPartMax) cl_sort_part(arr + plo, plen, cl_smem, one, t);
     __syncthreads();
   }
+  if (GAS_BKC_TMA_STORE && t == 0) asm volatile("cp.async.bulk.wait_group 0;" ::: "memory");  // part stores complete
 }
 
 // The rare arrays with an oversize part: a global-memory bitonic network over
