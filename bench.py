@@ -372,8 +372,8 @@ def main():
             kernel_hint = "k_pairs"
         elif 512 < n <= 1024 and os.environ.get("GAS_BUCKET", "1") != "0":
             # the sort1024 pipeline's kernel that takes a batch of this distribution (tools/launches.sh)
-            kernel_hint = {"uniform_bits": "k_s1_count", "spectra_intensity": "k_s1_count", "dup16": "k_s1_count",
-                           "special_mix": "k_s1_net"}.get(dist, "k_fixed_bucket1024")
+            kernel_hint = {"uniform_bits": "k_s1_count", "spectra_intensity": "k_s1_count", "dup16": "k_s1_split",
+                           "special_mix": "k_s1_split"}.get(dist, "k_fixed_bucket1024")
         else:
             kernel_hint = "k_fixed_warp" if n <= 1024 else "k_fixed_cta"
         n_desc = str(n)

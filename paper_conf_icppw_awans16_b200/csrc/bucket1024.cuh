@@ -231,10 +231,10 @@ __device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
 // ---- Control block of the 512 < n <= 1024 pipeline (sort1024.cuh): device
 // workspace of one gas_sort_arrays call, followed by an array-index list of
 // up to N entries.
-enum : uint32_t { kS1Bucket = 0, kS1Count = 1, kS1Network = 2 };
+enum : uint32_t { kS1Bucket = 0, kS1Count = 1, kS1Split = 2 };
 struct S1Ctl {
   uint32_t flag;      // the path that takes the whole batch (kS1*), written by the sampler
-  uint32_t nlist;     // arrays the counting-sort kernel hands to the network (zeroed by the sampler)
+  uint32_t nlist;     // arrays the counting-sort kernel hands to the split kernel (zeroed by the sampler)
 };
 // The list of nlist array indices follows the control block.
 __device__ __forceinline__ uint32_t* s1_list(S1Ctl* c) { return reinterpret_cast<uint32_t*>(c + 1); }

@@ -8,6 +8,7 @@
 #include "segsort.cuh"
 #include "bucket1024.cuh"
 #include "sort1024.cuh"
+#include "split1024.cuh"
 
 namespace gas_host {
 
@@ -73,7 +74,7 @@ cudaError_t launch_fixed_sort1024(uint32_t* d, int64_t N, int n, cudaStream_t s)
 
 
 // Default for large batches: the device-routed pipeline of sort1024.cuh
-// (sampler -> bucket kernel -> counting-sort kernel -> network kernel), 4
+// (sampler -> bucket kernel -> counting-sort kernel -> split kernel), 4
 // launches and 4 N + 8 bytes of stream-ordered workspace.
 template <bool VEC>
 cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
@@ -81,7 +82,9 @@ cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   cudaError_t e = ws_alloc(&ws, sizeof(gas::S1Ctl) + 4 * (size_t)N, s);
   if (e != cudaSuccess) return e;
   gas::S1Ctl* ctl = static_cast<gas::S1Ctl*>(ws);
-  gas::k_s1_sample<VEC><<<1, 1024, 0, s>>>(d, N, n, ctl);
+  const char* fv = std::getenv("GAS_S1_FORCE");  // tests / ablations: 0 bucket, 1 counting sort, 2 split kernel
+  const uint32_t force = fv && fv[0] ? (uint32_t)std::atoi(fv) : 0xFFFFFFFFu;
+  gas::k_s1_sample<VEC><<<1, 1024, 0, s>>>(d, N, n, ctl, force);
   e = cudaGetLastError();
   if (e == cudaSuccess) {
     auto k = VEC ? gas::k_fixed_bucket1024<true> : gas::k_fixed_bucket1024_any<false, true>;
@@ -104,13 +107,12 @@ cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
     }
   }
   if (e == cudaSuccess) {
-    auto k = gas::k_s1_net<VEC>;
-    constexpr int smem = gas::kS1NetBlock / 32 * 4096;
-    e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    auto k = gas::k_s1_split<VEC>;
+    e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kSpSmemBytes);
     if (e == cudaSuccess) {
-      const int grid = persistent_grid_smem(k, gas::kS1NetBlock, smem,
-                                            (N + gas::kS1NetBlock / 32 - 1) / (gas::kS1NetBlock / 32));
-      k<<<grid, gas::kS1NetBlock, smem, s>>>(d, N, n, 1u, ctl);
+      const int grid = persistent_grid_smem(k, gas::kSpBlock, gas::kSpSmemBytes,
+                                            (N + gas::kSpBlock / 32 - 1) / (gas::kSpBlock / 32));
+      k<<<grid, gas::kSpBlock, gas::kSpSmemBytes, s>>>(d, N, n, 1u, ctl);
       e = cudaGetLastError();
     }
   }

@@ -257,22 +257,38 @@ __global__ void __launch_bounds__(kS1Block, 1)
 //   3. k_s1_count: the counting sort over the whole batch when flag == count;
 //      special-heavy arrays go to a list; arrays failing its own check are
 //      finished by the network inline (rare).
-//   4. k_s1_net: the 1024-key network over the whole batch (flag == network)
-//      or over that list (its arrays are read from HBM a second time).
+//   4. k_s1_split (split1024.cuh): value buckets with special-value runs and
+//      equal-key runs, over the whole batch (flag == split: NaN / inf / ±0
+//      mixes, duplicate-heavy data) or over that list (its arrays are read
+//      from HBM a second time); its own leftovers take the network inline.
 // Kernels not chosen exit at once (a few microseconds each).
 
-// The class an array votes for: special-heavy sample -> network; finite values
-// whose 32-key sample fits the buckets -> bucket; else the counting sort.
+// The class an array votes for: special-heavy sample -> split; finite values
+// whose 32-key sample fits the buckets -> bucket; duplicate-heavy samples
+// whose repeated values each fill a bucket of their own -> split; else the
+// counting sort.
 __device__ __forceinline__ uint32_t s1_sample_special(uint32_t k0) {
   const bool special = ((k0 >> 23) & 0xFFu) == 0xFFu || k0 == 0x80000000u;  // inf / NaN / -0
   return __popc(__ballot_sync(0xffffffffu, special));
 }
 
+// Duplicate-heavy sample the split kernel's equal-key runs can take: some
+// value appears >= 3 times among the 32 sample keys, and every sample bucket
+// holds a single value (a bucket overflowing with two values would not fold).
+__device__ __forceinline__ bool bk_sample_dup(uint32_t k0, float vmin, float s) {
+  const uint32_t sb = bucket_bits(k0, vmin, s) - 0x4B000000u;
+  const uint32_t mv = __match_any_sync(0xffffffffu, k0);
+  const bool single = __all_sync(0xffffffffu, __match_any_sync(0xffffffffu, sb) == mv);
+  return single && __reduce_max_sync(0xffffffffu, __popc(mv)) >= 3;
+}
+
 // One block of 32 warps; warp w samples array floor(w N / 32). The block
-// writes the majority vote into ctl->flag and zeroes the list counter (no
-// other initialisation of the workspace is needed).
+// writes the majority vote into ctl->flag (or `force`, when <= kS1Split:
+// tests and ablations, GAS_S1_FORCE) and zeroes the list counter (no other
+// initialisation of the workspace is needed).
 template <bool VEC>
-__global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restrict__ d, int64_t N, int n, S1Ctl* ctl) {
+__global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restrict__ d, int64_t N, int n, S1Ctl* ctl,
+                                                           uint32_t force) {
   __shared__ uint32_t votes[3];
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
   if (threadIdx.x < 3) votes[threadIdx.x] = 0;
@@ -304,22 +320,22 @@ __global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restric
     const bool raw = umin > 0u && umax < 0x7F800000u;
     uint32_t cls;
     if (!raw && s1_sample_special(bk_sample_key<VEC>(k, lane)) >= 2) {
-      cls = kS1Network;
+      cls = kS1Split;
     } else {
       const bool finite = kmin > 0x007FFFFFu && kmax < 0xFF800000u;
       const float vmin = __uint_as_float(bits_from_key(kmin));
       const float range = __fsub_rn(__uint_as_float(bits_from_key(kmax)), vmin);
       const float s = __fdiv_rn((float)GAS_BK_TOP, range);
       bool ok = finite && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
-      if (ok) ok = bk_sample_ok(bk_sample_key<VEC>(k, lane), raw, vmin, s);
-      cls = ok ? kS1Bucket : kS1Count;
+      const uint32_t k0 = bk_sample_key<VEC>(k, lane);
+      cls = ok && bk_sample_ok(k0, raw, vmin, s) ? kS1Bucket : (ok && bk_sample_dup(k0, vmin, s) ? kS1Split : kS1Count);
     }
     if (lane == 0) atomicAdd(&votes[cls], 1u);
   }
   __syncthreads();
   if (threadIdx.x == 0) {
-    const uint32_t vb = votes[kS1Bucket], vc = votes[kS1Count], vn = votes[kS1Network];
-    ctl->flag = (vb >= vc && vb >= vn) ? kS1Bucket : (vc >= vn ? kS1Count : kS1Network);
+    const uint32_t vb = votes[kS1Bucket], vc = votes[kS1Count], vn = votes[kS1Split];
+    ctl->flag = force <= kS1Split ? force : (vb >= vc && vb >= vn) ? kS1Bucket : (vc >= vn ? kS1Count : kS1Split);
     ctl->nlist = 0;
   }
 }
@@ -373,34 +389,10 @@ __global__ void __launch_bounds__(kCwBlock, 1) k_s1_count(uint32_t* __restrict__
     umax = __reduce_max_sync(0xffffffffu, max(umax, k[31]));
     const bool raw = umin > 0u && umax < 0x7F800000u;
     if (!raw && s1_sample_special(bk_sample_key<VEC>(k, lane)) >= 2) {
-      s1_push(ctl->nlist, s1_list(ctl), a, lane);  // special-heavy: the network kernel takes it
+      s1_push(ctl->nlist, s1_list(ctl), a, lane);  // special-heavy: the split kernel takes it
       continue;
     }
     cw_sort_warp<VEC>(k, raw, umin, umax, 0u, arr, n, lane, cnt_sa, buf_sa, buf_ptr, one);
-  }
-}
-
-// 4. The 1024-key network (warp1024.cuh) over the whole batch (flag ==
-// network) or over the counting-sort kernel's list.
-constexpr int kS1NetBlock = 512;  // 16 warps per SM at <= 128 registers (the network's best)
-template <bool VEC>
-__global__ void __launch_bounds__(kS1NetBlock, 1) k_s1_net(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one,
-                                                           S1Ctl* ctl) {
-  extern __shared__ __align__(16) uint4 net_smem[];
-  const uint32_t flag = ctl->flag;
-  const int64_t count = flag == kS1Network ? N : (int64_t)ctl->nlist;
-  const uint32_t* list = s1_list(ctl);
-  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-  uint32_t* const scratch = reinterpret_cast<uint32_t*>(net_smem) + warp * 1024;
-  const int64_t nwarps = (int64_t)gridDim.x * (kS1NetBlock / 32);
-  for (int64_t i = (int64_t)blockIdx.x * (kS1NetBlock / 32) + warp; i < count; i += nwarps) {
-    const int64_t a = flag == kS1Network ? i : (int64_t)list[i];
-    uint32_t* const arr = d + a * (int64_t)n;
-    uint32_t k[32];
-    s1_load<VEC>(k, arr, n, lane);
-    if constexpr (VEC) bucket1024_fallback(k, reinterpret_cast<uint4*>(arr), n >> 2, lane, scratch, one);
-    else bucket1024_fallback_scalar(k, arr, n, lane, scratch, one);
-    __syncwarp();
   }
 }
 
