@@ -25,9 +25,10 @@
 // A negative normal value's bucket never exceeds b0 and a positive one's is
 // never below it (the map is monotone), so the rows above are in order. Runs
 // are attached to a neighbouring row in the bucket scan: -inf after row 1,
-// the zeros after the negative subnormals, +inf before the keys of row 62. Arrays without NaN / inf (the "plain"
-// path: duplicate-heavy data) use the 64 value buckets of bucket1024.cuh
-// over [min, max] with the same equal-run overflow rule.
+// the zeros after the negative subnormals, +inf before the keys of row 62.
+// Arrays without NaN / inf (the "plain" path: duplicate-heavy data) use the
+// 64 value buckets of bucket1024.cuh over [min, max] with the same equal-run
+// overflow rule.
 // Whatever is left — a row of more than 32 keys with two distinct keys, a
 // value range that overflows — is re-read (L2) and sorted by the 1024-key
 // network (warp1024.cuh). Correctness rests on the same monotone map as
@@ -81,11 +82,17 @@ __device__ __forceinline__ uint32_t pl_row(uint32_t bits, float vmin, float s) {
 }
 
 // Rank + scatter of one array's keys: the atomic returns the key's rank in
-// its row; keys of rank >= 32 are only counted (their row overflows), and so
-// are run keys (row >= 64).
+// its row; run keys (row >= 64) are only counted. A key of rank >= 32 does
+// not fit: its row is written as a run if all its keys are equal. On the
+// plain path (duplicate-heavy data: overflow is the rule) the key is compared
+// here with the row's slot 0 (stored by the rank-0 key in this or an earlier
+// group); the SP path, where overflow is rare, leaves it to
+// sp_overflow_mismatch (no per-key cost when no row overflows). Returns
+// whether one of this lane's keys differs.
 template <bool SP, bool VEC>
-__device__ __forceinline__ void sp_scatter(const uint32_t (&k)[32], int lane, int n, const SpMap& m, float vmin,
+__device__ __forceinline__ bool sp_scatter(const uint32_t (&k)[32], int lane, int n, const SpMap& m, float vmin,
                                            float s, uint32_t cnt_sa, uint32_t slot_sa) {
+  bool mis = false;
 #pragma unroll
   for (int g = 0; g < 32; g += 4) {
     uint32_t row[4], c[4];
@@ -94,30 +101,59 @@ __device__ __forceinline__ void sp_scatter(const uint32_t (&k)[32], int lane, in
       row[r - g] = SP ? sp_row(k[r], m) : pl_row(k[r], vmin, s);
       c[r - g] = atoms_inc_if(cw_valid<VEC>(r, lane, n), cnt_sa + row[r - g] * 4);
     }
+    uint32_t ra[4], kk[4];
+    bool ov[4];
 #pragma unroll
     for (int r = g; r < g + 4; ++r) {
-      const bool v = cw_valid<VEC>(r, lane, n) && (!SP || row[r - g] < 64u) && c[r - g] < 32u;
-      sts32_if(v, slot_sa + row[r - g] * (kSpRowWords * 4) + c[r - g] * 4, key_from_bits(k[r]));
+      const bool v = cw_valid<VEC>(r, lane, n) && (!SP || row[r - g] < 64u);
+      kk[r - g] = key_from_bits(k[r]);
+      ra[r - g] = slot_sa + row[r - g] * (kSpRowWords * 4);
+      sts32_if(v && c[r - g] < 32u, ra[r - g] + c[r - g] * 4, kk[r - g]);
+      ov[r - g] = v && c[r - g] >= 32u;
+    }
+    if (!SP && __any_sync(0xffffffffu, ov[0] || ov[1] || ov[2] || ov[3])) {
+      __syncwarp();  // slot 0 of every row touched so far is stored
+#pragma unroll
+      for (int j = 0; j < 4; ++j) {
+        uint32_t v = kk[j];  // slot 0 of the key's row when it overflowed, else the key itself
+        asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %1, 0;\n\t@q ld.shared.u32 %0, [%2];\n\t}"
+                     : "+r"(v) : "r"((uint32_t)ov[j]), "r"(ra[j]) : "memory");
+        mis |= v != kk[j];
+      }
     }
   }
+  return mis;
 }
 
-// Equal-key check of the overflowing rows (mask om0: rows 0..31, om1: rows
-// 32..63): every key of such a row must equal the row's slot 0. Returns
-// whether one of this lane's keys does not.
-template <bool SP, bool VEC>
+// SP path: every key of an overflowing row (masks om0: rows 0..31, om1: rows
+// 32..63) must equal the row's slot 0. Returns whether one of this lane's
+// keys does not.
+template <bool VEC>
 __device__ __forceinline__ bool sp_overflow_mismatch(const uint32_t (&k)[32], int lane, int n, const SpMap& m,
-                                                     float vmin, float s, uint32_t slot_sa, uint32_t om0,
-                                                     uint32_t om1) {
+                                                     uint32_t slot_sa, uint32_t om0, uint32_t om1) {
   bool bad = false;
 #pragma unroll
   for (int r = 0; r < 32; ++r) {
-    const uint32_t row = SP ? sp_row(k[r], m) : pl_row(k[r], vmin, s);
+    const uint32_t row = sp_row(k[r], m);
     const uint32_t bit = ((row < 32u ? om0 : om1) >> (row & 31u)) & 1u;
-    const bool over = cw_valid<VEC>(r, lane, n) && (!SP || row < 64u) && bit != 0u;
-    if (over) bad |= lds32(slot_sa + row * (kSpRowWords * 4)) != key_from_bits(k[r]);
+    const bool over = cw_valid<VEC>(r, lane, n) && row < 64u && bit != 0u;
+    const uint32_t kk = key_from_bits(k[r]);
+    uint32_t v = kk;
+    asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %1, 0;\n\t@q ld.shared.u32 %0, [%2];\n\t}"
+                 : "+r"(v) : "r"((uint32_t)over), "r"(slot_sa + row * (kSpRowWords * 4)) : "memory");
+    bad |= v != kk;
   }
   return bad;
+}
+
+// Writes `len` copies of key `val` at staged positions [st, st + len) (one
+// lane; 16-byte stores between the unaligned ends).
+__device__ __forceinline__ void sp_fill(uint32_t stage_sa, uint32_t st, uint32_t len, uint32_t val) {
+  uint32_t p = st;
+  const uint32_t e = st + len;
+  for (; p < e && (p & 3u); ++p) sts32(stage_sa + p * 4, val);
+  for (; p + 4 <= e; p += 4) sts128(stage_sa + p * 4, make_uint4(val, val, val, val));
+  for (; p < e; ++p) sts32(stage_sa + p * 4, val);
 }
 
 // The pipeline's split kernel: the whole batch when ctl->flag == kS1Split,
@@ -208,19 +244,18 @@ __global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__
       sts32(cnt_sa + 128 + lane * 4, 0u);
       if (lane < 4) sts32(cnt_sa + 256 + lane * 4, 0u);
       __syncwarp();
-      if (sp) sp_scatter<true, VEC>(k, lane, n, m, vmin, s, cnt_sa, slot_sa);
-      else sp_scatter<false, VEC>(k, lane, n, m, vmin, s, cnt_sa, slot_sa);
+      const bool mis = sp ? sp_scatter<true, VEC>(k, lane, n, m, vmin, s, cnt_sa, slot_sa)
+                          : sp_scatter<false, VEC>(k, lane, n, m, vmin, s, cnt_sa, slot_sa);
+      bad = __any_sync(0xffffffffu, mis);
       __syncwarp();
     }
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0, r_ninf = 0, r_nz = 0, r_pz = 0, r_pinf = 0;
     if (ok) {
       t0 = lds32(cnt_sa + lane * 4);
       t1 = lds32(cnt_sa + 128 + lane * 4);
-      const uint32_t om0 = __ballot_sync(0xffffffffu, t0 > 32u), om1 = __ballot_sync(0xffffffffu, t1 > 32u);
-      if (om0 | om1) {  // overflowing rows: runs if all their keys are equal, else the network
-        const bool mis = sp ? sp_overflow_mismatch<true, VEC>(k, lane, n, m, vmin, s, slot_sa, om0, om1)
-                            : sp_overflow_mismatch<false, VEC>(k, lane, n, m, vmin, s, slot_sa, om0, om1);
-        bad = __any_sync(0xffffffffu, mis);
+      if (sp) {
+        const uint32_t om0 = __ballot_sync(0xffffffffu, t0 > 32u), om1 = __ballot_sync(0xffffffffu, t1 > 32u);
+        if (om0 | om1) bad = __any_sync(0xffffffffu, sp_overflow_mismatch<VEC>(k, lane, n, m, slot_sa, om0, om1));
       }
       if (sp) {
         r_ninf = lds32(cnt_sa + 256);
@@ -263,21 +298,39 @@ __global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__
 #pragma unroll
           for (int q = 0; q < 32; ++q) k[q] = kPadKey;
         }
-        const uint32_t tl = over ? 1u : tb;  // an overflowing row: only its slot 0
+        const uint32_t tl = min(tb, 32u);
 #pragma unroll
         for (int q = 0; q < 8; ++q) lds128_if(4u * q < tl, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
-        const uint32_t rep = k[0];  // an overflowing row: all its keys equal its slot 0
+        const uint32_t rep = k[0];  // an overflowing row: all its keys must equal its slot 0
+        if (__any_sync(0xffffffffu, over)) {
+          uint32_t lo = k[0], hi = k[0];
+#pragma unroll
+          for (int q = 1; q < 31; q += 2) {
+            lo = __vimin3_u32(lo, k[q], k[q + 1]);
+            hi = __vimax3_u32(hi, k[q], k[q + 1]);
+          }
+          if (__any_sync(0xffffffffu, over && (lo != hi || k[31] != lo))) {
+            bad = true;
+            break;
+          }
+        }
         if (rho) rep0 = rep;
         else rep1 = rep;
         __syncwarp();  // rows 32..63 are drained before any output is staged over them
-        if (__any_sync(0xffffffffu, !over && tb >= 2u)) sortn_bk<32>(k, one);
+        const bool keys = !over && tb != 0u;
+        if (__any_sync(0xffffffffu, keys)) {  // else every row of this round is empty or a run
+          if (__any_sync(0xffffffffu, keys && tb >= 2u)) sortn_bk<32>(k, one);
 #pragma unroll
-        for (int q = 0; q < 32; ++q) sts32_if(!over && (uint32_t)q < tb, ob + q * 4, k[q]);
+          for (int q = 0; q < 32; ++q) sts32_if(keys && (uint32_t)q < tb, ob + q * 4, k[q]);
+        }
       }
     }
     if (!bad) {
       // ---- runs: equal-key overflow rows, then (SP) -inf, -0, +0, +inf
-      uint32_t om0 = __ballot_sync(0xffffffffu, t0 > 32u), om1 = __ballot_sync(0xffffffffu, t1 > 32u);
+      // each lane writes its own overflow rows' runs; runs longer than 256 keys are written by the warp
+      if (t1 > 32u && t1 <= 256u) sp_fill(stage_sa, base1, t1, rep1);
+      if (t0 > 32u && t0 <= 256u) sp_fill(stage_sa, base0, t0, rep0);
+      uint32_t om0 = __ballot_sync(0xffffffffu, t0 > 256u), om1 = __ballot_sync(0xffffffffu, t1 > 256u);
       while (om0 | om1) {
         const bool hi = om0 == 0u;
         const int owner = __ffs(hi ? om1 : om0) - 1;
