@@ -7,6 +7,8 @@
 // memory and gathered by position after the sort; keys and payloads are
 // written back in place through a rank-order staging buffer (coalesced).
 // Algorithmic bytes: 16n per array (keys and payloads read and written once).
+// `list` (or nullptr): sort only the arrays it names (count, then indices) —
+// the leftovers of the bucket kernel of pairs1024.cuh.
 #pragma once
 #include <cstdint>
 
@@ -28,7 +30,8 @@ struct PairsCfg {
 
 template <int KPT, int G, int W>
 __global__ void __launch_bounds__(PairsCfg<KPT, G, W>::TPB)
-    k_pairs(uint32_t* __restrict__ keys, uint32_t* __restrict__ vals, int64_t N, int n) {
+    k_pairs(uint32_t* __restrict__ keys, uint32_t* __restrict__ vals, int64_t N, int n,
+            const uint32_t* __restrict__ list) {
   using C = PairsCfg<KPT, G, W>;
   constexpr int P = C::P, TH = C::TH;
   extern __shared__ __align__(16) unsigned char pairs_smem[];
@@ -39,9 +42,10 @@ __global__ void __launch_bounds__(PairsCfg<KPT, G, W>::TPB)
   uint32_t* vs = reinterpret_cast<uint32_t*>(base);           // payloads, input order
   uint4* ks = reinterpret_cast<uint4*>(base + P * 4);         // rank-order staging (swizzled chunks)
   uint64_t* xs = reinterpret_cast<uint64_t*>(base + P * 8);   // cross-warp exchange (W > 1)
+  if (list) N = list[0];  // a worklist (pairs1024.cuh): count, then array indices
   for (int64_t a0 = (int64_t)blockIdx.x * C::GROUPS; a0 < N; a0 += (int64_t)gridDim.x * C::GROUPS) {
-    const int64_t a = a0 + grp;
-    const bool valid = a < N;
+    const bool valid = a0 + grp < N;
+    const int64_t a = !valid ? 0 : (list ? (int64_t)list[1 + a0 + grp] : a0 + grp);
     const int64_t off = (valid ? a : 0) * (int64_t)n;
     uint64_t k[KPT];
 #pragma unroll
