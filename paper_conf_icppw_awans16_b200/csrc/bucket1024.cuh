@@ -231,7 +231,7 @@ __device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
 // ---- Control block of the 512 < n <= 1024 pipeline (sort1024.cuh): device
 // workspace of one gas_sort_arrays call, followed by an array-index list of
 // up to N entries.
-enum : uint32_t { kS1Bucket = 0, kS1Count = 1, kS1Split = 2 };
+enum : uint32_t { kS1Bucket = 0, kS1Count = 1, kS1Split = 2, kS1KeyLin = 3 };
 struct S1Ctl {
   uint32_t flag;      // the path that takes the whole batch (kS1*), written by the sampler
   uint32_t nlist;     // arrays the counting-sort kernel hands to the split kernel (zeroed by the sampler)
@@ -241,6 +241,20 @@ __device__ __forceinline__ uint32_t* s1_list(S1Ctl* c) { return reinterpret_cast
 __device__ __forceinline__ const uint32_t* s1_list(const S1Ctl* c) { return reinterpret_cast<const uint32_t*>(c + 1); }
 __device__ __forceinline__ void s1_push(uint32_t& count, uint32_t* list, int64_t a, int lane) {
   if (lane == 0) list[atomicAdd(&count, 1u)] = (uint32_t)a;
+}
+
+// Key-linear bucket map (KL kernels): b(key) = umulhi(key - kmin, M) with
+//     M = min(2^32 - 1, floor(2^38 / (kmax - kmin + 1)))   (computed rounding down),
+// so 0 <= b <= 63 (x M < 2^38 for x <= kmax - kmin) and b is non-decreasing in
+// the key. Keys are the totalOrder keys (ordered_key.cuh), or the raw bits of
+// an all-positive finite array, so NaN, infinities and ±0 need no special
+// case: the order of the keys is the order of the output (C-1).
+// Key-linear buckets are uniform over the bit patterns (BASELINE.json
+// uniform_bits), where value-linear buckets put nearly every key into bucket 0.
+__device__ __forceinline__ uint32_t kl_mult(uint32_t kmin, uint32_t kmax) {
+  const float den = __fadd_ru(__uint2float_ru(kmax - kmin), 1.0f);  // >= range + 1
+  const float q = __fdiv_rz(274877906944.0f, den);                   // <= 2^38 / (range + 1)
+  return q >= 4294967040.0f ? 0xFFFFFFFFu : __float2uint_rz(q);
 }
 
 #ifndef GAS_S1_PRED  // sample keys in one value bucket that send an array to the counting sort
@@ -303,10 +317,14 @@ __device__ __forceinline__ bool bk_sample_ok(uint32_t k0, bool raw, float vmin, 
 //     first size_b network outputs are bucket b sorted in both rounds.
 //     Outputs are staged at slot words kBkStageWord + base_b + i.
 //  5. coalesced in-place store (key -> bits for non-raw arrays).
-template <bool PIPE>
+// KL: the key-linear map (kl_mult) instead of the value map: any bit pattern
+// (NaN, infinities, ±0) takes the bucket path; only an overflowing bucket sends
+// the array to the fallback. Non-raw arrays stage bits, so every array leaves
+// through the TMA bulk store. (The pipeline's kS1KeyLin kernel.)
+template <bool PIPE, bool KL = false>
 __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     k_fixed_bucket1024(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one, const S1Ctl* ctl) {
-  if (PIPE && ctl->flag != kS1Bucket) return;  // pipeline (sort1024.cuh): another kernel takes this batch
+  if (PIPE && ctl->flag != (KL ? kS1KeyLin : kS1Bucket)) return;  // pipeline (sort1024.cuh): another kernel takes this batch
   extern __shared__ __align__(16) uint4 bk_smem[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
@@ -359,6 +377,8 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     umax = __reduce_max_sync(0xffffffffu, max(umax, k[31]));
     const bool raw = umin > 0u && umax < 0x7F800000u;  // every value positive and finite
     bool use_buckets = true;
+    float vmin = 0.0f, s = 0.0f;
+    uint32_t klo = umin, mk = 0;  // KL: key minimum and multiplier
     if (!raw) {  // min / max in key space; an infinity or NaN (either sign) -> fallback
       uint32_t kmin = 0xFFFFFFFFu, kmax = 0u;
 #pragma unroll
@@ -369,14 +389,23 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       }
       kmin = __reduce_min_sync(0xffffffffu, kmin);
       kmax = __reduce_max_sync(0xffffffffu, kmax);
-      use_buckets = kmin > 0x007FFFFFu && kmax < 0xFF800000u;
-      umin = bits_from_key(kmin);
-      umax = bits_from_key(kmax);
+      if constexpr (KL) {
+        klo = kmin;
+        umax = kmax;
+      } else {
+        use_buckets = kmin > 0x007FFFFFu && kmax < 0xFF800000u;
+        umin = bits_from_key(kmin);
+        umax = bits_from_key(kmax);
+      }
     }
-    const float vmin = __uint_as_float(umin), vmax = __uint_as_float(umax);
-    const float range = __fsub_rn(vmax, vmin);
-    const float s = __fdiv_rn((float)GAS_BK_TOP, range);
-    use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
+    if constexpr (KL) {
+      mk = kl_mult(klo, umax);
+    } else {
+      vmin = __uint_as_float(umin);
+      const float range = __fsub_rn(__uint_as_float(umax), vmin);
+      s = __fdiv_rn((float)GAS_BK_TOP, range);
+      use_buckets = use_buckets && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
+    }
     uint32_t t0 = 0, t1 = 0, base0 = 0, base1 = 0;
     if (use_buckets) {
       // lane l owns buckets l (row l) and l + 32 (row 32 + l)
@@ -385,7 +414,33 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       __syncwarp();
       // ---- rank + scatter: the atomic returns the key's slot address
       // (in groups of GAS_BK_GROUP keys: the atomics of a group are in flight together)
-      if (raw) {
+      if constexpr (KL) {
+        if (raw) {
+#pragma unroll
+          for (int g = 0; g < 32; g += GAS_BK_GROUP) {
+            uint32_t sa[GAS_BK_GROUP];
+#pragma unroll
+            for (int r = g; r < g + GAS_BK_GROUP; ++r)
+              sa[r - g] = atoms_add4_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, __umulhi(k[r] - klo, mk) * 4u + cnt_sa);
+#pragma unroll
+            for (int r = g; r < g + GAS_BK_GROUP; ++r)
+              sts32_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, min(sa[r - g], slot_last), k[r]);
+          }
+        } else {
+#pragma unroll
+          for (int g = 0; g < 32; g += GAS_BK_GROUP) {
+            uint32_t sa[GAS_BK_GROUP], kk[GAS_BK_GROUP];
+#pragma unroll
+            for (int r = g; r < g + GAS_BK_GROUP; ++r) {
+              kk[r - g] = key_from_bits(k[r]);
+              sa[r - g] = atoms_add4_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, __umulhi(kk[r - g] - klo, mk) * 4u + cnt_sa);
+            }
+#pragma unroll
+            for (int r = g; r < g + GAS_BK_GROUP; ++r)
+              sts32_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, min(sa[r - g], slot_last), kk[r - g]);
+          }
+        }
+      } else if (raw) {
 #pragma unroll
         for (int g = 0; g < 32; g += GAS_BK_GROUP) {
           uint32_t sa[GAS_BK_GROUP];

@@ -98,7 +98,6 @@ __device__ __forceinline__ uint32_t cw_kl_shift(uint32_t kmin, uint32_t kmax) {
   const int bits = 32 - __clz(dk);  // bit length of the range
   return bits > 11 ? (uint32_t)(bits - 11) : 0u;
 }
-
 // Key r of this lane lies inside the array: VEC, chunk layout (key r is
 // element 4 (lane + 32 (r/4)) + r%4; n > 512 so chunks 0..3 always exist);
 // scalar layout (key r is element lane + 32 r).

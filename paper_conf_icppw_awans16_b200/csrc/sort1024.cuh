@@ -257,6 +257,9 @@ __global__ void __launch_bounds__(kS1Block, 1)
 //   3. k_s1_count: the counting sort over the whole batch when flag == count;
 //      special-heavy arrays go to a list; arrays failing its own check are
 //      finished by the network inline (rare).
+//   2b. k_fixed_bucket1024<PIPE, KL = true>: the same kernel with the
+//      key-linear map (flag == keylin: the sample does not fit value buckets
+//      but fits key-linear ones, e.g. arrays of arbitrary bit patterns).
 //   4. k_s1_split (split1024.cuh): value buckets with special-value runs and
 //      equal-key runs, over the whole batch (flag == split: NaN / inf / ±0
 //      mixes, duplicate-heavy data) or over that list (its arrays are read
@@ -282,18 +285,28 @@ __device__ __forceinline__ bool bk_sample_dup(uint32_t k0, float vmin, float s) 
   return single && __reduce_max_sync(0xffffffffu, __popc(mv)) >= 3;
 }
 
-// One block of 32 warps; warp w samples array floor(w N / 32). The block
-// writes the majority vote into ctl->flag (or `force`, when <= kS1Split:
-// tests and ablations, GAS_S1_FORCE) and zeroes the list counter (no other
-// initialisation of the workspace is needed).
+// One block of 32 warps; warp w samples array floor(w N / 32) and counts, in
+// shared memory, the exact bucket sizes that array gets under the value map
+// (bk kernel) and the key-linear map (KL kernel). The batch goes to
+//   the value buckets   when >= 26 of 32 sampled arrays fit them (<= 32 keys
+//                       per bucket; an overflowing array costs the bucket
+//                       attempt plus the 1024-key network, ~1.8x),
+//   the key-linear ones when >= 27 of 32 fit those,
+//   else the split kernel or the counting sort, by the majority of the
+//   sampled arrays' votes (special-heavy or duplicate-heavy -> split).
+// `force` (<= kS1KeyLin; tests and ablations, GAS_S1_FORCE) overrides the
+// choice. The block also zeroes the list counter (no other initialisation of
+// the workspace is needed).
 template <bool VEC>
 __global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restrict__ d, int64_t N, int n, S1Ctl* ctl,
                                                            uint32_t force) {
-  __shared__ uint32_t votes[3];
+  __shared__ uint32_t votes[4];  // [0] value buckets fit, [1] key-linear buckets fit, [2] count, [3] split
+  __shared__ uint32_t hist[32][128];  // per warp: 64 value-bucket sizes, 64 key-linear bucket sizes
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  if (threadIdx.x < 3) votes[threadIdx.x] = 0;
+  if (threadIdx.x < 4) votes[threadIdx.x] = 0;
   __syncthreads();
-  if ((int64_t)w < N) {
+  const int64_t S = N < 32 ? N : 32;  // arrays sampled
+  if ((int64_t)w < S) {
     const int64_t a = (N <= 32) ? w : (int64_t)(((__int128)w * N) >> 5);
     const uint32_t* arr = d + a * (int64_t)n;
     uint32_t k[32];
@@ -318,24 +331,43 @@ __global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restric
     kmin = __reduce_min_sync(0xffffffffu, kmin);
     kmax = __reduce_max_sync(0xffffffffu, kmax);
     const bool raw = umin > 0u && umax < 0x7F800000u;
-    uint32_t cls;
-    if (!raw && s1_sample_special(bk_sample_key<VEC>(k, lane)) >= 2) {
-      cls = kS1Split;
-    } else {
-      const bool finite = kmin > 0x007FFFFFu && kmax < 0xFF800000u;
-      const float vmin = __uint_as_float(bits_from_key(kmin));
-      const float range = __fsub_rn(__uint_as_float(bits_from_key(kmax)), vmin);
-      const float s = __fdiv_rn((float)GAS_BK_TOP, range);
-      bool ok = finite && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
-      const uint32_t k0 = bk_sample_key<VEC>(k, lane);
-      cls = ok && bk_sample_ok(k0, raw, vmin, s) ? kS1Bucket : (ok && bk_sample_dup(k0, vmin, s) ? kS1Split : kS1Count);
+    const bool finite = kmin > 0x007FFFFFu && kmax < 0xFF800000u;
+    const float vmin = __uint_as_float(bits_from_key(kmin));
+    const float range = __fsub_rn(__uint_as_float(bits_from_key(kmax)), vmin);
+    const float s = __fdiv_rn((float)GAS_BK_TOP, range);
+    const bool ok = finite && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
+    const uint32_t mk = kl_mult(kmin, kmax);
+    // exact bucket sizes of this array under both maps (the kernels' own maps)
+    uint32_t* const h = hist[w];
+#pragma unroll
+    for (int j = 0; j < 4; ++j) h[lane + 32 * j] = 0u;
+    __syncwarp();
+#pragma unroll
+    for (int r = 0; r < 32; ++r) {
+      if (cw_valid<VEC>(r, lane, n)) {
+        if (ok) atomicAdd(&h[bucket_bits(k[r], vmin, s) - 0x4B000000u], 1u);
+        atomicAdd(&h[64u + __umulhi(key_from_bits(k[r]) - kmin, mk)], 1u);
+      }
     }
-    if (lane == 0) atomicAdd(&votes[cls], 1u);
+    __syncwarp();
+    const bool vfit = ok && __reduce_max_sync(0xffffffffu, max(h[lane], h[lane + 32])) <= 32u;
+    const bool kfit = VEC && __reduce_max_sync(0xffffffffu, max(h[64 + lane], h[96 + lane])) <= 32u;
+    const uint32_t k0 = bk_sample_key<VEC>(k, lane);
+    const bool to_split = (!raw && s1_sample_special(k0) >= 2) || (ok && bk_sample_dup(k0, vmin, s));
+    if (lane == 0) {
+      if (vfit) atomicAdd(&votes[0], 1u);
+      if (kfit) atomicAdd(&votes[1], 1u);
+      atomicAdd(&votes[to_split ? 3 : 2], 1u);
+    }
   }
   __syncthreads();
   if (threadIdx.x == 0) {
-    const uint32_t vb = votes[kS1Bucket], vc = votes[kS1Count], vn = votes[kS1Split];
-    ctl->flag = force <= kS1Split ? force : (vb >= vc && vb >= vn) ? kS1Bucket : (vc >= vn ? kS1Count : kS1Split);
+    uint32_t best;
+    if ((int64_t)votes[0] * 32 >= 26 * S) best = kS1Bucket;
+    else if ((int64_t)votes[1] * 32 >= 27 * S) best = kS1KeyLin;
+    else best = votes[3] > votes[2] ? kS1Split : kS1Count;
+    if (force <= kS1KeyLin) best = force;
+    ctl->flag = (!VEC && best == kS1KeyLin) ? kS1Count : best;  // the key-linear kernel takes 16-byte rows only
     ctl->nlist = 0;
   }
 }
