@@ -101,6 +101,10 @@ __device__ __forceinline__ void bar_cta(uint32_t bar) {
 // words before the first and after the last 16-byte boundary are stored one by
 // one). Thread 0 waits for the previous store's reads before the group's first
 // row write of the next array; the kernel waits for completion before exiting.
+#ifndef GAS_BKC_VOTE_MERGE
+#define GAS_BKC_VOTE_MERGE 1
+#endif
+constexpr uint32_t kBkcOverflow = 0xFFFFFFFFu;  // a warp's scan total when one of its buckets overflowed (totals < 2^31)
 template <int W, int WR, bool VEC, int RV = 16, bool TMA = (GAS_BKC_TMA_STORE != 0)>
 __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int n, unsigned char* sm, uint32_t one,
                                                 int t, uint32_t bar) {
@@ -212,8 +216,12 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
     bar_cta<WR>(bar);
     t0 = (lds32(cnt_sa + t * 4) - row0) >> 2;
     t1 = (lds32(cnt_sa + (T + t) * 4) - row1) >> 2;
-    if constexpr (WR > 1) use_buckets = group_and(t0 <= 32u && t1 <= 32u, bar);
+    // overflow vote and bucket bases share one barrier: a warp whose buckets
+    // fit posts its scan total, one that overflows posts kBkcOverflow
+    // (GAS_BKC_VOTE_MERGE=0: a separate bar.red.and vote first)
+    if constexpr (WR > 1 && !GAS_BKC_VOTE_MERGE) use_buckets = group_and(t0 <= 32u && t1 <= 32u, bar);
     else use_buckets = __all_sync(0xffffffffu, t0 <= 32u && t1 <= 32u);
+    uint32_t x = 0, before = 0, total = 0;
     if (use_buckets) {
 #pragma unroll
       for (int j = 0; j < 3; ++j) {
@@ -221,14 +229,29 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
         sts32_if(((t1 + j) & 3u) != 0u, row1 + (t1 + j) * 4, kPadKey);
       }
       // bucket bases: exclusive scan of the 2T bucket sizes (two 16-bit halves)
-      uint32_t x = t0 | (t1 << 16);
+      x = t0 | (t1 << 16);
 #pragma unroll
       for (int m = 1; m < 32; m <<= 1) {
         const uint32_t y = __shfl_up_sync(0xffffffffu, x, m);
         if (lane >= m) x += y;
       }
-      uint32_t before = 0, total = __shfl_sync(0xffffffffu, x, 31);
-      if constexpr (WR > 1) {
+      total = __shfl_sync(0xffffffffu, x, 31);
+    }
+    if constexpr (WR > 1 && GAS_BKC_VOTE_MERGE) {
+      uint32_t* const part = red + 64;
+      if (lane == 31) part[warp] = use_buckets ? x : kBkcOverflow;
+      group_sync(bar);  // also publishes the pads
+      total = 0;
+#pragma unroll
+      for (int w = 0; w < WR; ++w) {
+        const uint32_t pw = part[w];
+        use_buckets = use_buckets && pw != kBkcOverflow;
+        before += (w < warp) ? pw : 0u;
+        total += pw;
+      }
+    }
+    if (use_buckets) {
+      if constexpr (WR > 1 && !GAS_BKC_VOTE_MERGE) {
         uint32_t* const part = red + 64;
         if (lane == 31) part[warp] = x;
         group_sync(bar);  // also publishes the pads
