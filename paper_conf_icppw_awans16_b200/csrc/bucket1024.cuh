@@ -231,10 +231,13 @@ __device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
 // ---- Control block of the 512 < n <= 1024 pipeline (sort1024.cuh): device
 // workspace of one gas_sort_arrays call, followed by an array-index list of
 // up to N entries.
-enum : uint32_t { kS1Bucket = 0, kS1Count = 1, kS1Split = 2, kS1KeyLin = 3 };
+enum : uint32_t { kS1Bucket = 0, kS1Count = 1, kS1Split = 2, kS1KeyLin = 3, kS1Cdf = 4 };
+constexpr int kCdfEntries = 512;  // batch CDF table: one entry per (sign, exponent) of the key, i.e. key >> 23
 struct S1Ctl {
   uint32_t flag;      // the path that takes the whole batch (kS1*), written by the sampler
   uint32_t nlist;     // arrays the counting-sort kernel hands to the split kernel (zeroed by the sampler)
+  uint32_t pad[2];
+  uint2 cdf[kCdfEntries];  // (A, B) of the batch CDF map (cdf_bucket), written by the sampler
 };
 // The list of nlist array indices follows the control block.
 __device__ __forceinline__ uint32_t* s1_list(S1Ctl* c) { return reinterpret_cast<uint32_t*>(c + 1); }
@@ -242,6 +245,30 @@ __device__ __forceinline__ const uint32_t* s1_list(const S1Ctl* c) { return rein
 __device__ __forceinline__ void s1_push(uint32_t& count, uint32_t* list, int64_t a, int lane) {
   if (lane == 0) list[atomicAdd(&count, 1u)] = (uint32_t)a;
 }
+
+// Batch-CDF bucket map (MAP = kMapCdf): the sampler estimates, from the keys
+// of its 32 sampled arrays (S keys), the distribution function of the batch at
+// the 512 binade boundaries of the key space (e = key >> 23: sign and
+// exponent) and writes, per entry e with c_e sampled keys and P_e sampled keys
+// below it,
+//     A_e = min(2^32 - 1, floor(P_e 2^32 / S)),   B_e = floor(c_e 2^16 / S).
+// A key's bucket is b = (A_e + m' B_e) >> 26 with m' = the top 16 mantissa
+// bits: the estimated distribution function at the key, linear inside a
+// binade, times 64. For every key, 0 <= b <= 63 and b is non-decreasing in the
+// key, whatever the table holds as long as it was built this way:
+// A_e + (2^16 - 1) B_e < (P_e + c_e) 2^32 / S and, being an integer, is at most
+// A_{e+1}. Arrays drawn from the batch's distribution (spectra intensities:
+// log-normal-like, BASELINE.json spectra_intensity) then get ~n/64 keys per
+// bucket, as flat data does under the value map. This is the paper's
+// "sampling according to the distribution" (§9; splitters from a
+// sample, Alg. 1) moved from one array to the batch.
+__device__ __forceinline__ uint32_t cdf_bucket_addr(uint32_t kk, uint32_t tbl_sa, uint32_t cnt_sa) {
+  uint32_t a, b;
+  asm volatile("ld.shared.v2.u32 {%0, %1}, [%2];" : "=r"(a), "=r"(b) : "r"(tbl_sa + (kk >> 23) * 8u) : "memory");
+  const uint32_t u = a + ((kk >> 7) & 0xFFFFu) * b;
+  return cnt_sa + (u >> 26) * 4u;
+}
+enum : int { kMapValue = 0, kMapKeyLin = 1, kMapCdf = 2 };
 
 // Key-linear bucket map (KL kernels): b(key) = umulhi(key - kmin, M) with
 //     M = min(2^32 - 1, floor(2^38 / (kmax - kmin + 1)))   (computed rounding down),
@@ -321,12 +348,24 @@ __device__ __forceinline__ bool bk_sample_ok(uint32_t k0, bool raw, float vmin, 
 // (NaN, infinities, ±0) takes the bucket path; only an overflowing bucket sends
 // the array to the fallback. Non-raw arrays stage bits, so every array leaves
 // through the TMA bulk store. (The pipeline's kS1KeyLin kernel.)
-template <bool PIPE, bool KL = false>
+// MAP = kMapCdf: the batch-CDF map (cdf_bucket_addr); the table (4 KB) is
+// copied into shared memory after the per-warp areas.
+template <bool PIPE, int MAP = kMapValue>
 __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
     k_fixed_bucket1024(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one, const S1Ctl* ctl) {
-  if (PIPE && ctl->flag != (KL ? kS1KeyLin : kS1Bucket)) return;  // pipeline (sort1024.cuh): another kernel takes this batch
+  constexpr bool KL = MAP != kMapValue;  // keys (not values) are bucketed: every bit pattern takes the bucket path
+  if (PIPE && ctl->flag != (MAP == kMapCdf ? kS1Cdf : (MAP == kMapKeyLin ? kS1KeyLin : kS1Bucket))) return;
   extern __shared__ __align__(16) uint4 bk_smem[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const uint32_t tbl_sa = (uint32_t)__cvta_generic_to_shared(bk_smem) + (kBkBlock / 32) * kBkWarpBytes;
+  if constexpr (MAP == kMapCdf) {
+    for (int e = threadIdx.x; e < kCdfEntries; e += kBkBlock) {
+      const uint2 v = ctl->cdf[e];
+      asm volatile("st.shared.v2.u32 [%0], {%1, %2};" ::"r"(tbl_sa + e * 8u), "r"(v.x), "r"(v.y) : "memory");
+    }
+    __syncthreads();
+  }
+  const uint32_t tbl_raw = tbl_sa + 256u * 8u;  // raw (all positive) arrays: key >> 23 = (bits >> 23) + 256
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(bk_smem) + warp * kBkWarpBytes;
   const uint32_t cnt_sa = wsa;                               // counter of bucket b at cnt_sa + b*4
   const uint32_t slot_sa = wsa + kBkCntBytes;                // slot (p, b) at slot_sa + (36 b + p)*4
@@ -398,8 +437,10 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         umax = bits_from_key(kmax);
       }
     }
-    if constexpr (KL) {
+    if constexpr (MAP == kMapKeyLin) {
       mk = kl_mult(klo, umax);
+    } else if constexpr (MAP == kMapCdf) {
+      (void)mk;
     } else {
       vmin = __uint_as_float(umin);
       const float range = __fsub_rn(__uint_as_float(umax), vmin);
@@ -414,7 +455,33 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       __syncwarp();
       // ---- rank + scatter: the atomic returns the key's slot address
       // (in groups of GAS_BK_GROUP keys: the atomics of a group are in flight together)
-      if constexpr (KL) {
+      if constexpr (MAP == kMapCdf) {
+        if (raw) {
+#pragma unroll
+          for (int g = 0; g < 32; g += GAS_BK_GROUP) {
+            uint32_t sa[GAS_BK_GROUP];
+#pragma unroll
+            for (int r = g; r < g + GAS_BK_GROUP; ++r)
+              sa[r - g] = atoms_add4_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, cdf_bucket_addr(k[r], tbl_raw, cnt_sa));
+#pragma unroll
+            for (int r = g; r < g + GAS_BK_GROUP; ++r)
+              sts32_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, min(sa[r - g], slot_last), k[r]);
+          }
+        } else {
+#pragma unroll
+          for (int g = 0; g < 32; g += GAS_BK_GROUP) {
+            uint32_t sa[GAS_BK_GROUP], kk[GAS_BK_GROUP];
+#pragma unroll
+            for (int r = g; r < g + GAS_BK_GROUP; ++r) {
+              kk[r - g] = key_from_bits(k[r]);
+              sa[r - g] = atoms_add4_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, cdf_bucket_addr(kk[r - g], tbl_sa, cnt_sa));
+            }
+#pragma unroll
+            for (int r = g; r < g + GAS_BK_GROUP; ++r)
+              sts32_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, min(sa[r - g], slot_last), kk[r - g]);
+          }
+        }
+      } else if constexpr (KL) {
         if (raw) {
 #pragma unroll
           for (int g = 0; g < 32; g += GAS_BK_GROUP) {

@@ -74,7 +74,7 @@ cudaError_t launch_fixed_sort1024(uint32_t* d, int64_t N, int n, cudaStream_t s)
 
 
 // Default for large batches: the device-routed pipeline of sort1024.cuh
-// (sampler -> bucket kernel -> key-linear bucket kernel (16-byte rows) -> counting-sort kernel -> split kernel), 5 (4)
+// (sampler -> bucket kernel -> key-linear and batch-CDF bucket kernels (16-byte rows) -> counting-sort kernel -> split kernel), 6 (4)
 // launches and 4 N + 8 bytes of stream-ordered workspace.
 template <bool VEC>
 cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
@@ -82,7 +82,7 @@ cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   cudaError_t e = ws_alloc(&ws, sizeof(gas::S1Ctl) + 4 * (size_t)N, s);
   if (e != cudaSuccess) return e;
   gas::S1Ctl* ctl = static_cast<gas::S1Ctl*>(ws);
-  const char* fv = std::getenv("GAS_S1_FORCE");  // tests / ablations: 0 bucket, 1 counting sort, 2 split kernel, 3 key-linear buckets
+  const char* fv = std::getenv("GAS_S1_FORCE");  // tests / ablations: 0 bucket, 1 counting sort, 2 split kernel, 3 key-linear buckets, 4 batch-CDF buckets
   const uint32_t force = fv && fv[0] ? (uint32_t)std::atoi(fv) : 0xFFFFFFFFu;
   gas::k_s1_sample<VEC><<<1, 1024, 0, s>>>(d, N, n, ctl, force);
   e = cudaGetLastError();
@@ -96,13 +96,15 @@ cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
       e = cudaGetLastError();
     }
   }
-  if (VEC && e == cudaSuccess) {
-    auto k = gas::k_fixed_bucket1024<true, true>;
-    e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kBkSmemBytes);
+  // key-linear and batch-CDF bucket kernels (16-byte rows only)
+  for (int map = gas::kMapKeyLin; VEC && map <= gas::kMapCdf && e == cudaSuccess; ++map) {
+    auto k = map == gas::kMapKeyLin ? gas::k_fixed_bucket1024<true, gas::kMapKeyLin>
+                                    : gas::k_fixed_bucket1024<true, gas::kMapCdf>;
+    const int smem = gas::kBkSmemBytes + (map == gas::kMapCdf ? gas::kCdfEntries * 8 : 0);
+    e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
     if (e == cudaSuccess) {
-      const int grid = persistent_grid_smem(k, gas::kBkBlock, gas::kBkSmemBytes,
-                                            (N + gas::kBkBlock / 32 - 1) / (gas::kBkBlock / 32));
-      k<<<grid, gas::kBkBlock, gas::kBkSmemBytes, s>>>(d, N, n, 1u, ctl);
+      const int grid = persistent_grid_smem(k, gas::kBkBlock, smem, (N + gas::kBkBlock / 32 - 1) / (gas::kBkBlock / 32));
+      k<<<grid, gas::kBkBlock, smem, s>>>(d, N, n, 1u, ctl);
       e = cudaGetLastError();
     }
   }
@@ -127,7 +129,7 @@ cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
     }
   }
   const cudaError_t f = cudaFreeAsync(ws, s);  // stream-ordered: after the kernels
-  if (e == cudaSuccess) launch_counter() += VEC ? 5 : 4;
+  if (e == cudaSuccess) launch_counter() += VEC ? 6 : 4;
   return e != cudaSuccess ? e : f;
 }
 
@@ -149,7 +151,7 @@ cudaError_t dispatch_1024(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   if (bucket_enabled() && sort1024_enabled()) {
     const char* mv = std::getenv("GAS_SORT1024_MODE");  // a forced branch runs in the fused kernel
     if ((!mv || std::atoi(mv) == 0) && N >= s1_pipeline_min() && N < (int64_t(1) << 32))
-      return launch_s1_pipeline<VEC>(d, N, n, s);  // counts its own 4 or 5 launches
+      return launch_s1_pipeline<VEC>(d, N, n, s);  // counts its own 6 (4) launches
     launch_counter() += 1;
     return launch_fixed_sort1024<VEC>(d, N, n, s);
   }

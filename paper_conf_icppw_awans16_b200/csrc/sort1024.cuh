@@ -285,31 +285,44 @@ __device__ __forceinline__ bool bk_sample_dup(uint32_t k0, float vmin, float s) 
   return single && __reduce_max_sync(0xffffffffu, __popc(mv)) >= 3;
 }
 
-// One block of 32 warps; warp w samples array floor(w N / 32) and counts, in
-// shared memory, the exact bucket sizes that array gets under the value map
-// (bk kernel) and the key-linear map (KL kernel). The batch goes to
-//   the value buckets   when >= 26 of 32 sampled arrays fit them (<= 32 keys
-//                       per bucket; an overflowing array costs the bucket
-//                       attempt plus the 1024-key network, ~1.8x),
-//   the key-linear ones when >= 27 of 32 fit those,
+// One block of 32 warps; warp w samples array floor(w N / 32).
+//  1. every sampled key goes into a 512-bin histogram of key >> 23 (sign and
+//     exponent of the totalOrder key); threads 0..511 scan it and write the
+//     batch-CDF table of cdf_bucket_addr (bucket1024.cuh) to ctl->cdf;
+//  2. each warp counts, in shared memory, the exact bucket sizes its array
+//     gets under the value map (bk kernel), the key-linear map (KL kernel)
+//     and the batch-CDF map (CDF kernel).
+// The batch goes to
+//   the value buckets     when >= 26 of 32 sampled arrays fit them (<= 32 keys
+//                         per bucket; an overflowing array costs the bucket
+//                         attempt plus the 1024-key network, ~1.8x),
+//   the key-linear ones   when >= 27 fit those,
+//   the batch-CDF ones    when >= 27 fit those,
 //   else the split kernel or the counting sort, by the majority of the
 //   sampled arrays' votes (special-heavy or duplicate-heavy -> split).
-// `force` (<= kS1KeyLin; tests and ablations, GAS_S1_FORCE) overrides the
+// `force` (<= kS1Cdf; tests and ablations, GAS_S1_FORCE) overrides the
 // choice. The block also zeroes the list counter (no other initialisation of
 // the workspace is needed).
 template <bool VEC>
 __global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restrict__ d, int64_t N, int n, S1Ctl* ctl,
                                                            uint32_t force) {
-  __shared__ uint32_t votes[4];  // [0] value buckets fit, [1] key-linear buckets fit, [2] count, [3] split
-  __shared__ uint32_t hist[32][128];  // per warp: 64 value-bucket sizes, 64 key-linear bucket sizes
+  __shared__ uint32_t votes[5];  // [0] value fit, [1] key-linear fit, [2] count, [3] split, [4] batch-CDF fit
+  __shared__ uint32_t hist[32][192];  // per warp: value-bucket, key-linear and batch-CDF bucket sizes
+  __shared__ uint32_t h512[kCdfEntries];
+  __shared__ __align__(8) uint2 tbl[kCdfEntries];
+  __shared__ uint32_t part[kCdfEntries / 32];
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  if (threadIdx.x < 4) votes[threadIdx.x] = 0;
+  if (threadIdx.x < 5) votes[threadIdx.x] = 0;
+  if (threadIdx.x < kCdfEntries) h512[threadIdx.x] = 0;
   __syncthreads();
   const int64_t S = N < 32 ? N : 32;  // arrays sampled
-  if ((int64_t)w < S) {
-    const int64_t a = (N <= 32) ? w : (int64_t)(((__int128)w * N) >> 5);
-    const uint32_t* arr = d + a * (int64_t)n;
-    uint32_t k[32];
+  const bool active = (int64_t)w < S;
+  const int64_t a = (N <= 32) ? w : (int64_t)(((__int128)w * N) >> 5);
+  const uint32_t* arr = d + (active ? a : 0) * (int64_t)n;
+  uint32_t k[32];
+  uint32_t* const h = hist[w];
+  // ---- 1. each sampled array: exact bucket sizes under the value and key-linear maps
+  if (active) {
 #pragma unroll
     for (int r = 0; r < 32; ++r) {
       const bool v = cw_valid<VEC>(r, lane, n);
@@ -337,21 +350,24 @@ __global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restric
     const float s = __fdiv_rn((float)GAS_BK_TOP, range);
     const bool ok = finite && range > 0.0f && range <= 3.402823466e38f && s <= 3.402823466e38f;
     const uint32_t mk = kl_mult(kmin, kmax);
-    // exact bucket sizes of this array under both maps (the kernels' own maps)
-    uint32_t* const h = hist[w];
 #pragma unroll
-    for (int j = 0; j < 4; ++j) h[lane + 32 * j] = 0u;
+    for (int j = 0; j < 6; ++j) h[lane + 32 * j] = 0u;
     __syncwarp();
+    if (ok) {
 #pragma unroll
-    for (int r = 0; r < 32; ++r) {
-      if (cw_valid<VEC>(r, lane, n)) {
-        if (ok) atomicAdd(&h[bucket_bits(k[r], vmin, s) - 0x4B000000u], 1u);
-        atomicAdd(&h[64u + __umulhi(key_from_bits(k[r]) - kmin, mk)], 1u);
-      }
+      for (int r = 0; r < 32; ++r)
+        if (cw_valid<VEC>(r, lane, n)) atomicAdd(&h[bucket_bits(k[r], vmin, s) - 0x4B000000u], 1u);
     }
     __syncwarp();
     const bool vfit = ok && __reduce_max_sync(0xffffffffu, max(h[lane], h[lane + 32])) <= 32u;
-    const bool kfit = VEC && __reduce_max_sync(0xffffffffu, max(h[64 + lane], h[96 + lane])) <= 32u;
+    bool kfit = false;  // counted only when the value buckets do not fit (the sampler is on the critical path)
+    if (VEC && !vfit) {
+#pragma unroll
+      for (int r = 0; r < 32; ++r)
+        if (cw_valid<VEC>(r, lane, n)) atomicAdd(&h[64u + __umulhi(key_from_bits(k[r]) - kmin, mk)], 1u);
+      __syncwarp();
+      kfit = __reduce_max_sync(0xffffffffu, max(h[64 + lane], h[96 + lane])) <= 32u;
+    }
     const uint32_t k0 = bk_sample_key<VEC>(k, lane);
     const bool to_split = (!raw && s1_sample_special(k0) >= 2) || (ok && bk_sample_dup(k0, vmin, s));
     if (lane == 0) {
@@ -361,13 +377,63 @@ __global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restric
     }
   }
   __syncthreads();
+  uint32_t best = kS1Count;
+  if ((int64_t)votes[0] * 32 >= 26 * S) best = kS1Bucket;
+  else if ((int64_t)votes[1] * 32 >= 27 * S) best = kS1KeyLin;
+  if (force <= kS1Cdf) best = force;
+  // ---- 2. (only when neither map fits, or forced) the batch-CDF table from all
+  // sampled keys, then each sampled array's bucket sizes under it (block-uniform branch)
+  const bool want_cdf = force <= kS1Cdf ? force == kS1Cdf : (best == kS1Count && VEC);
+  if (want_cdf) {
+    if (active) {
+#pragma unroll
+      for (int r = 0; r < 32; ++r)
+        if (cw_valid<VEC>(r, lane, n)) atomicAdd(&h512[key_from_bits(k[r]) >> 23], 1u);
+    }
+    __syncthreads();
+    // exclusive scan of the 512 bins (16 warps), then (A_e, B_e) of cdf_bucket_addr
+    uint32_t cnt = 0, total = 0;
+    if (threadIdx.x < kCdfEntries) {
+      cnt = h512[threadIdx.x];
+      uint32_t x = cnt;
+#pragma unroll
+      for (int m = 1; m < 32; m <<= 1) {
+        const uint32_t y = __shfl_up_sync(0xffffffffu, x, m);
+        if (lane >= m) x += y;
+      }
+      if (lane == 31) part[w] = x;
+      h512[threadIdx.x] = x - cnt;  // exclusive prefix inside the warp
+    }
+    __syncthreads();
+    if (threadIdx.x < kCdfEntries) {
+      uint32_t before = 0;
+#pragma unroll
+      for (int i = 0; i < kCdfEntries / 32; ++i) {
+        before += i < w ? part[i] : 0u;
+        total += part[i];
+      }
+      const uint64_t P = before + h512[threadIdx.x], T = total ? total : 1u;
+      const uint64_t A = (P << 32) / T;
+      const uint2 e = make_uint2(A > 0xFFFFFFFFull ? 0xFFFFFFFFu : (uint32_t)A, (uint32_t)(((uint64_t)cnt << 16) / T));
+      tbl[threadIdx.x] = e;
+      ctl->cdf[threadIdx.x] = e;
+    }
+    __syncthreads();
+    if (active) {
+      const uint32_t tsa = (uint32_t)__cvta_generic_to_shared(tbl);
+#pragma unroll
+      for (int r = 0; r < 32; ++r)
+        if (cw_valid<VEC>(r, lane, n)) atomicAdd(&h[128u + (cdf_bucket_addr(key_from_bits(k[r]), tsa, 0u) >> 2)], 1u);
+      __syncwarp();
+      const bool cfit = __reduce_max_sync(0xffffffffu, max(h[128 + lane], h[160 + lane])) <= 32u;
+      if (lane == 0 && cfit) atomicAdd(&votes[4], 1u);
+    }
+    __syncthreads();
+    if (force > kS1Cdf && (int64_t)votes[4] * 32 >= 27 * S) best = kS1Cdf;
+  }
   if (threadIdx.x == 0) {
-    uint32_t best;
-    if ((int64_t)votes[0] * 32 >= 26 * S) best = kS1Bucket;
-    else if ((int64_t)votes[1] * 32 >= 27 * S) best = kS1KeyLin;
-    else best = votes[3] > votes[2] ? kS1Split : kS1Count;
-    if (force <= kS1KeyLin) best = force;
-    ctl->flag = (!VEC && best == kS1KeyLin) ? kS1Count : best;  // the key-linear kernel takes 16-byte rows only
+    if (force > kS1Cdf && best == kS1Count) best = votes[3] > votes[2] ? kS1Split : kS1Count;
+    ctl->flag = (!VEC && (best == kS1KeyLin || best == kS1Cdf)) ? kS1Count : best;  // those kernels take 16-byte rows only
     ctl->nlist = 0;
   }
 }

@@ -102,9 +102,68 @@ def test_bucket_capacity_edges(keylin, count):
 
 def test_natural_routing_uniform_bits(monkeypatch):
     """Unforced: a uniform_bits batch of the pipeline's size is voted to the
-    key-linear kernel (5 launches: sampler + four path kernels), bit-exact."""
+    key-linear kernel (6 launches: sampler + five path kernels), bit-exact."""
     monkeypatch.delenv("GAS_S1_FORCE", raising=False)
     host = datagen.fixed("uniform_bits", 9500, 0, 20000, 1000)
     before = gas.launch_count()
     check(host)
-    assert gas.launch_count() - before == 5
+    assert gas.launch_count() - before == 6
+
+
+# ---- the batch-CDF bucket kernel (k_fixed_bucket1024<PIPE, kMapCdf>): buckets from
+# the distribution function the sampler estimates over its 32 sampled arrays
+
+@pytest.fixture
+def cdf(monkeypatch):
+    monkeypatch.setenv("GAS_S1_FORCE", "4")
+    monkeypatch.setenv("GAS_S1_PIPELINE_MIN", "1")
+
+
+@pytest.mark.parametrize("dist", DISTS)
+@pytest.mark.parametrize("n", [516, 776, 1000, 1024])
+def test_cdf_forced_every_distribution(cdf, dist, n):
+    check(datagen.fixed(dist, 9600 + n, 0, 400, n))
+
+
+@pytest.mark.parametrize("N", [1, 2, 31, 33, 5000])
+def test_cdf_forced_batch_sizes(cdf, N):
+    """Fewer arrays than the sampler's 32 (the table comes from all of them) and
+    batches far larger than the sample (arrays the table never saw)."""
+    check(datagen.fixed("spectra_intensity", 9650 + N, 0, N, 1000))
+
+
+def test_cdf_forced_mixed_batch(cdf):
+    """Arrays from different distributions in one batch: the sampled table fits
+    none of them well; buckets overflow and take the network, every array exact."""
+    parts = [datagen.fixed(d, 9660, 0, 300, 1000) for d in ("spectra_intensity", "uniform_bits", "special_mix", "dup16")]
+    host = np.concatenate(parts)
+    host = np.ascontiguousarray(host[np.random.default_rng(3).permutation(host.shape[0])])
+    check(host)
+
+
+def test_cdf_forced_edges(cdf):
+    rng = np.random.default_rng(78)
+    cases = [
+        # keys in binades the sampled arrays never held (table entries with no samples)
+        np.concatenate([datagen.fixed("spectra_intensity", 9670, 0, 40, 1000),
+                        (rng.integers(0, 2**32, size=(24, 1000))).astype(np.uint32)]),
+        # every key equal; the two extreme keys; NaN / inf / zeros
+        np.stack([np.full(1000, 0x3F800000, dtype=np.uint32),
+                  np.concatenate([[0xFFFFFFFF, 0x7FFFFFFF], rng.integers(0, 2**32, size=998)]).astype(np.uint32),
+                  np.concatenate([[0x7F800000, 0xFF800000, 0, 0x80000000, 0x7FC00001, 0xFFC00001] * 10,
+                                  rng.integers(0x3F800000, 0x40000000, size=940)]).astype(np.uint32)]),
+    ]
+    for c in cases:
+        for row in c:
+            rng.shuffle(row)
+        check(np.ascontiguousarray(c))
+
+
+def test_natural_routing_spectra_intensity(monkeypatch):
+    """Unforced: log-normal-like intensities overflow value and key-linear
+    buckets but fit the batch-CDF buckets; the sampler picks that kernel."""
+    monkeypatch.delenv("GAS_S1_FORCE", raising=False)
+    host = datagen.fixed("spectra_intensity", 9680, 0, 20000, 1000)
+    before = gas.launch_count()
+    check(host)
+    assert gas.launch_count() - before == 6

@@ -197,7 +197,7 @@ def test_pipeline_routes_mixed_batches(parts):
     host = _mixed_batch(parts)
     before = gas.launch_count()
     check(host)
-    assert gas.launch_count() - before == 5  # sampler + four path kernels (16-byte rows)
+    assert gas.launch_count() - before == 6  # sampler + five path kernels (16-byte rows)
 
 
 @pytest.mark.parametrize("n", [513, 999, 1000, 1024])

@@ -228,4 +228,4 @@ def test_natural_routing(parts):
     host = np.ascontiguousarray(host[np.random.default_rng(5).permutation(host.shape[0])])
     before = gas.launch_count()
     check(host)
-    assert gas.launch_count() - before == 5
+    assert gas.launch_count() - before == 6
