@@ -36,6 +36,17 @@ cudaError_t launch_fixed_bucket512(uint32_t* d, int64_t N, int n, cudaStream_t s
 }
 
 
+// Bucket-then-network kernel for 128 < n <= 256 with aligned rows (bucket512.cuh, half a warp per array).
+cudaError_t launch_fixed_bucket256(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  const cudaError_t attr = cudaFuncSetAttribute(gas::k_fixed_bucket256, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                                gas::kBk2SmemBytes);
+  if (attr != cudaSuccess) return attr;
+  const int grid = persistent_grid_smem(gas::k_fixed_bucket256, gas::kBk2Block, gas::kBk2SmemBytes,
+                                        (N + 2 * GAS_BK2_WARPS - 1) / (2 * GAS_BK2_WARPS));
+  gas::k_fixed_bucket256<<<grid, gas::kBk2Block, gas::kBk2SmemBytes, s>>>(d, N, n, 1u);
+  return cudaGetLastError();
+}
+
 template <bool VEC>
 cudaError_t dispatch_small(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   switch (size_class(n)) {
@@ -46,7 +57,9 @@ cudaError_t dispatch_small(uint32_t* d, int64_t N, int n, cudaStream_t s) {
     case 32: return launch_fixed_warp<32, 1, VEC>(d, N, n, s);
     case 64: return launch_fixed_warp<32, 2, VEC>(d, N, n, s);
     case 128: return launch_fixed_warp<32, 4, VEC>(d, N, n, s);
-    case 256: return launch_fixed_warp<32, 8, VEC>(d, N, n, s);
+    case 256:
+      if (VEC && bucket_enabled() && n > 128) return launch_fixed_bucket256(d, N, n, s);
+      return launch_fixed_warp<32, 8, VEC>(d, N, n, s);
     case 512:
       if (VEC && bucket_enabled()) return launch_fixed_bucket512(d, N, n, s);
       return launch_fixed_warp<32, 16, VEC>(d, N, n, s);

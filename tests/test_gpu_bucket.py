@@ -317,6 +317,42 @@ def test_bucket512_many_arrays_and_unaligned():
     np.testing.assert_array_equal(gpu_sort_fixed(host, lead=1), expect)  # network class (scalar path)
 
 
+# ---- bucket512.cuh: k_fixed_bucket256, 128 < n <= 256 (16-byte rows), half a warp per array, 16 buckets
+
+@pytest.mark.parametrize("n", [132, 200, 252, 256])
+@pytest.mark.parametrize("dist", ["paper_uniform", "spectra_mz", "sorted", "reverse", "spectra_intensity",
+                                  "dup16", "special_mix", "uniform_bits"])
+def test_bucket256_distributions(dist, n):
+    host = datagen.fixed(dist, 7120, 0, 701, n)  # odd count: the last warp's second half has no array
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("N", [1, 2, 3, 47, 48, 49])
+def test_bucket256_batch_sizes(N):
+    host = datagen.fixed("paper_uniform", 7121 + N, 0, N, 248)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("count", [32, 33])
+def test_bucket256_capacity_edge(count):
+    """A bucket of exactly 32 keys fits; 33 sends both arrays of the warp to the network."""
+    rng = np.random.default_rng(400 + count)
+    rows = [spread_array(250, rng, heavy_bucket=5, heavy_count=count,
+                         heavy_values=5.0 + rng.uniform(-0.49, 0.49, size=count), top=15) for _ in range(63)]
+    host = np.stack(rows)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
+
+
+def test_bucket256_mixed_paths_in_one_warp():
+    """Neighbouring arrays (the two halves of a warp) where one overflows or holds NaN and the other does not."""
+    host = datagen.fixed("paper_uniform", 7130, 0, 4000, 240)
+    host[1::2] = datagen.fixed("dup16", 7131, 0, len(host[1::2]), 240)
+    host[::7] = datagen.fixed("special_mix", 7132, 0, len(host[::7]), 240)
+    expect = oracle_sorted(host)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=4), expect)
+    np.testing.assert_array_equal(gpu_sort_fixed(host, lead=1), expect)  # network class (scalar path)
+
+
 @pytest.mark.parametrize("n", [513, 515, 700, 999, 1021, 1023])
 @pytest.mark.parametrize("dist", ["paper_uniform", "special_mix", "dup16", "spectra_intensity"])
 def test_bucket_warp_unaligned(dist, n):
