@@ -7,8 +7,9 @@
 // own bucket idea (§4.1) one level up:
 //  1. CTA c loads its slice [c n/C, (c+1) n/C) and its key min / max; the
 //     cluster's min / max come from the C CTAs' shared memory over DSMEM;
-//  2. each CTA counts its keys into 256 key-linear coarse bins
-//     f = (key - kmin) >> sh; every CTA then reads all C histograms over DSMEM
+//  2. each CTA counts its keys into 256 coarse bins (value-linear over the
+//     array's range when every value is finite, else key-linear
+//     f = (key - kmin) >> sh); every CTA then reads all C histograms over DSMEM
 //     and derives the same partition: part p = the bins whose exclusive prefix
 //     lies in [p n/C, (p+1) n/C) (monotone in the key), its array positions
 //     [start_p, start_{p+1}) and this CTA's write offset in it;
@@ -102,9 +103,15 @@ __device__ __forceinline__ void cl_sort_part(uint32_t* arr, int len, unsigned ch
 // One cluster of C CTAs per array (persistent over arrays; the cluster shape
 // is a launch attribute); `fail` (count, then indices) receives the arrays
 // with a part longer than the CTA class holds.
-template <int W, int WR, int C, int MAXN>
-__global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
-    k_cluster_sort(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one, uint32_t* __restrict__ fail) {
+// PART (the two-kernel path, cluster_partition_sort): steps 1-3 only; CTA 0
+// writes the C part boundaries of array a to parts[a C .. a C + C - 1]
+// (element offsets into the batch: a CSR of N C parts) and lists the array in
+// `fail` when a part exceeds kClPartMaxOff; no dynamic shared memory.
+constexpr int kClPartMaxOff = 16384;  // longest part the offsets classes take
+template <int W, int WR, int C, int MAXN, bool PART = false>
+__global__ void __launch_bounds__(32 * WR, PART ? 3 : bkc_min_blocks<WR>())
+    k_cluster_sort(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one, uint32_t* __restrict__ fail,
+                   int64_t* __restrict__ parts) {
   using G = ClCfg<W, WR, C, MAXN>;
   constexpr int T = G::T, NB = G::NB, NB2 = G::NB2, KPT1 = G::KPT1;
   extern __shared__ __align__(16) unsigned char cl_smem[];
@@ -154,10 +161,21 @@ __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
     const int bits = 32 - __clz(kmax - kmin);
     constexpr int LNB = NB == 256 ? 8 : 9;
     const uint32_t sh = bits > LNB ? (uint32_t)(bits - LNB) : 0u;
+    // coarse bin of a key: value-linear over [vmin, vmax] when every value is
+    // finite (the map of bucket1024.cuh: uniform values give uniform bins, and
+    // few lanes of a warp hit one counter), else key-linear; both monotone
+    const float vmin = __uint_as_float(bits_from_key(kmin));
+    const float vrange = __fsub_rn(__uint_as_float(bits_from_key(kmax)), vmin);
+    const float vs = __fdiv_rn((float)(NB - 1), vrange);
+    const bool vmap = kmin > 0x007FFFFFu && kmax < 0xFF800000u && vrange > 0.0f && vrange <= 3.402823466e38f &&
+                      vs <= 3.402823466e38f;
+    auto bin = [&](uint32_t kk) -> uint32_t {
+      return vmap ? bucket_bits(bits_from_key(kk), vmin, vs) - 0x4B000000u : (kk - kmin) >> sh;
+    };
     // ---- 2. coarse histogram, then the partition from all C histograms
 #pragma unroll
     for (int r = 0; r < KPT1; ++r)
-      if (t + T * r < sl) atomicAdd(&hist[(k[r] - kmin) >> sh], 1u);
+      if (t + T * r < sl) atomicAdd(&hist[bin(k[r])], 1u);
     cl.sync();  // every CTA's histogram is final
     // thread t < NB2 owns bins 2t, 2t + 1: total count g and the count in lower CTAs
     uint32_t g[2] = {0u, 0u}, pre[2] = {0u, 0u};
@@ -216,22 +234,33 @@ __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
 #pragma unroll
     for (int r = 0; r < KPT1; ++r) {
       if (t + T * r < sl) {
-        const uint32_t pos = atomicAdd(&binpos[(k[r] - kmin) >> sh], 1u);  // 256 counters: little contention
+        const uint32_t pos = atomicAdd(&binpos[bin(k[r])], 1u);
         arr[pos] = bits_from_key(k[r]);
       }
     }
     cl.sync();  // every part is complete in memory (barrier.cluster arrive.release / wait.acquire) (and no peer still reads this CTA's hist / kmm)
-    // ---- 4. sort part c in place
-    const int plo = (int)pstart[c], plen = (int)pstart[c + 1] - plo;
-    if (c == 0 && t == 0) {  // every CTA holds the same pstart: CTA 0 lists the array once
-      bool over = false;
-      for (int p = 0; p < C; ++p) over |= pstart[p + 1] - pstart[p] > (uint32_t)G::CAP;
-      if (over) fail[1 + atomicAdd(&fail[0], 1u)] = (uint32_t)a;
+    if constexpr (PART) {
+      if (c == 0 && t < C) parts[a * C + t] = a * (int64_t)n + pstart[t];
+      if (c == 0 && t == 0) {
+        bool over = false;
+        for (int p = 0; p < C; ++p) over |= pstart[p + 1] - pstart[p] > (uint32_t)kClPartMaxOff;
+        if (over) fail[1 + atomicAdd(&fail[0], 1u)] = (uint32_t)a;
+      }
+      __syncthreads();  // pstart is rewritten by the next array
+    } else {
+      // ---- 4. sort part c in place
+      const int plo = (int)pstart[c], plen = (int)pstart[c + 1] - plo;
+      if (c == 0 && t == 0) {  // every CTA holds the same pstart: CTA 0 lists the array once
+        bool over = false;
+        for (int p = 0; p < C; ++p) over |= pstart[p + 1] - pstart[p] > (uint32_t)G::CAP;
+        if (over) fail[1 + atomicAdd(&fail[0], 1u)] = (uint32_t)a;
+      }
+      if (plen <= G::CAP) cl_sort_part<W, WR>(arr + plo, plen, cl_smem, one, t);
+      __syncthreads();
     }
-    if (plen <= G::CAP) cl_sort_part<W, WR>(arr + plo, plen, cl_smem, one, t);
-    __syncthreads();
   }
-  if (GAS_BKC_TMA_STORE && t == 0) asm volatile("cp.async.bulk.wait_group 0;" ::: "memory");  // part stores complete
+  if (PART && blockIdx.x == 0 && t == 0) parts[N * C] = N * (int64_t)n;  // the CSR's closing offset
+  if (!PART && GAS_BKC_TMA_STORE && t == 0) asm volatile("cp.async.bulk.wait_group 0;" ::: "memory");  // part stores complete
 }
 
 // The rare arrays with an oversize part: a global-memory bitonic network over

@@ -156,6 +156,69 @@ bool env_check() {
 
 }  // namespace
 
+namespace gas_host {
+
+// The variable-length (CSR) sort: per-class launches forked over side streams.
+cudaError_t offsets_sort(uint32_t* d, const int64_t* off, int64_t N, int32_t max_len, cudaStream_t s) {
+  // 9 window counters for the bucket classes' dynamic scheduling (72 bytes per call)
+  unsigned long long* ctr = nullptr;
+  if (max_len > 256) {
+    void* p = nullptr;
+    cudaError_t e = ws_alloc(&p, kCounters * sizeof(unsigned long long), s);
+    if (e == cudaSuccess) e = cudaMemsetAsync(p, 0, kCounters * sizeof(unsigned long long), s);
+    if (e != cudaSuccess) return e;
+    ctr = static_cast<unsigned long long*>(p);
+  }
+  // every exit below frees the counters on `s`, after the work that uses them
+  auto release = [&](cudaError_t e) -> cudaError_t {
+    if (ctr) {
+      const cudaError_t f = cudaFreeAsync(ctr, s);
+      if (e == cudaSuccess) e = f;
+    }
+    return e;
+  };
+  // size classes: 2, 4, ..., 2048 (len in (P/2, P]), then (2048, 3072] and (3072, 4096]
+  const int32_t classes[] = {2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288, 16384};
+  const int32_t lower[] = {1, 2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288};
+  int nclass = 0;
+  while (nclass < 17 && lower[nclass] < max_len) ++nclass;
+  // The class launches are independent (disjoint arrays). With K > 1 they are
+  // forked over K streams (largest classes first) so that each persistent
+  // launch's last wave overlaps the next launches instead of idling SMs; the
+  // caller's stream waits for all of them (CUDA-graph capture follows the
+  // fork/join). GAS_OFFSETS_STREAMS=1 restores one stream.
+  SideStreams* ss = nullptr;
+  if (offsets_streams() > 1 && nclass > 1) {
+    const cudaError_t e = side_streams_for(s, &ss);
+    if (e != cudaSuccess) return release(e);
+  }
+  if (!ss) {
+    for (int c = 0; c < nclass; ++c) {
+      const cudaError_t e = dispatch_offsets_class(classes[c], d, off, N, ctr, s);
+      if (e != cudaSuccess) return release(e);
+      launch_counter() += 1;
+    }
+    return release(cudaSuccess);
+  }
+  std::lock_guard<std::mutex> lock(ss->mu);
+  const int K = offsets_streams();
+  cudaError_t e = cudaEventRecord(ss->fork, s);
+  for (int i = 0; i < K && e == cudaSuccess; ++i) e = cudaStreamWaitEvent(ss->s[i], ss->fork, 0);
+  for (int c = nclass - 1, i = 0; c >= 0 && e == cudaSuccess; --c, ++i) {
+    e = dispatch_offsets_class(classes[c], d, off, N, ctr, ss->s[i % K]);
+    if (e == cudaSuccess) launch_counter() += 1;
+  }
+  // always join (also after an error) so that the caller's stream never races ahead
+  for (int i = 0; i < K; ++i) {
+    const cudaError_t r = cudaEventRecord(ss->join[i], ss->s[i]);
+    const cudaError_t w = r == cudaSuccess ? cudaStreamWaitEvent(s, ss->join[i], 0) : r;
+    if (e == cudaSuccess) e = w;
+  }
+  return release(e);
+}
+
+}  // namespace gas_host
+
 extern "C" {
 
 gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len, cudaStream_t stream) {
@@ -196,62 +259,8 @@ gas_status gas_sort_arrays_offsets(float* d_data, const int64_t* d_offsets, int6
     if (e != cudaSuccess) return cuda_fail(e);
     if (h) return GAS_ERROR_INVALID_VALUE;
   }
-  uint32_t* d = reinterpret_cast<uint32_t*>(d_data);
-  // 9 window counters for the bucket classes' dynamic scheduling (72 bytes per call)
-  unsigned long long* ctr = nullptr;
-  if (max_array_len > 256) {
-    void* p = nullptr;
-    cudaError_t e = ws_alloc(&p, kCounters * sizeof(unsigned long long), stream);
-    if (e == cudaSuccess) e = cudaMemsetAsync(p, 0, kCounters * sizeof(unsigned long long), stream);
-    if (e != cudaSuccess) return cuda_fail(e);
-    ctr = static_cast<unsigned long long*>(p);
-  }
-  // every exit below frees the counters on `stream`, after the work that uses them
-  auto release = [&](cudaError_t e) -> gas_status {
-    if (ctr) {
-      const cudaError_t f = cudaFreeAsync(ctr, stream);
-      if (e == cudaSuccess) e = f;
-    }
-    return e == cudaSuccess ? GAS_SUCCESS : cuda_fail(e);
-  };
-  // size classes: 2, 4, ..., 2048 (len in (P/2, P]), then (2048, 3072] and (3072, 4096]
-  const int32_t classes[] = {2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288, 16384};
-  const int32_t lower[] = {1, 2, 4, 8, 16, 32, 64, 128, 256, 512, 1024, 2048, 3072, 4096, 6144, 8192, 12288};
-  int nclass = 0;
-  while (nclass < 17 && lower[nclass] < max_array_len) ++nclass;
-  // The class launches are independent (disjoint arrays). With K > 1 they are
-  // forked over K streams (largest classes first) so that each persistent
-  // launch's last wave overlaps the next launches instead of idling SMs; the
-  // caller's stream waits for all of them (CUDA-graph capture follows the
-  // fork/join). GAS_OFFSETS_STREAMS=1 restores one stream.
-  SideStreams* ss = nullptr;
-  if (offsets_streams() > 1 && nclass > 1) {
-    const cudaError_t e = side_streams_for(stream, &ss);
-    if (e != cudaSuccess) return release(e);
-  }
-  if (!ss) {
-    for (int c = 0; c < nclass; ++c) {
-      const cudaError_t e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, ctr, stream);
-      if (e != cudaSuccess) return release(e);
-      launch_counter() += 1;
-    }
-    return release(cudaSuccess);
-  }
-  std::lock_guard<std::mutex> lock(ss->mu);
-  const int K = offsets_streams();
-  cudaError_t e = cudaEventRecord(ss->fork, stream);
-  for (int i = 0; i < K && e == cudaSuccess; ++i) e = cudaStreamWaitEvent(ss->s[i], ss->fork, 0);
-  for (int c = nclass - 1, i = 0; c >= 0 && e == cudaSuccess; --c, ++i) {
-    e = dispatch_offsets_class(classes[c], d, d_offsets, num_arrays, ctr, ss->s[i % K]);
-    if (e == cudaSuccess) launch_counter() += 1;
-  }
-  // always join (also after an error) so that the caller's stream never races ahead
-  for (int i = 0; i < K; ++i) {
-    const cudaError_t r = cudaEventRecord(ss->join[i], ss->s[i]);
-    const cudaError_t w = r == cudaSuccess ? cudaStreamWaitEvent(stream, ss->join[i], 0) : r;
-    if (e == cudaSuccess) e = w;
-  }
-  return release(e);
+  const cudaError_t e = offsets_sort(reinterpret_cast<uint32_t*>(d_data), d_offsets, num_arrays, max_array_len, stream);
+  return e == cudaSuccess ? GAS_SUCCESS : cuda_fail(e);
 }
 
 gas_status gas_sort_pairs(float* d_keys, uint32_t* d_values, int64_t num_arrays, int32_t array_len,

@@ -112,6 +112,8 @@ cudaError_t dispatch_fixed_small(bool vec, uint32_t* d, int64_t N, int n, cudaSt
 cudaError_t dispatch_fixed_1024(bool vec, uint32_t* d, int64_t N, int n, cudaStream_t s);   // 512 < n <= 1024
 cudaError_t dispatch_fixed_cta(bool vec, uint32_t* d, int64_t N, int n, cudaStream_t s);    // 1024 < n <= 16384
 cudaError_t dispatch_fixed_cluster(bool vec, uint32_t* d, int64_t N, int n, cudaStream_t s);  // 16384 < n <= 65536
+// The variable-length sort (gas_api.cu; also the second pass of the two-kernel cluster path)
+cudaError_t offsets_sort(uint32_t* d, const int64_t* off, int64_t N, int32_t max_len, cudaStream_t s);
 cudaError_t dispatch_offsets_class(int32_t P, uint32_t* d, const int64_t* off, int64_t N, unsigned long long* ctr,
                                    cudaStream_t s);
 cudaError_t dispatch_pairs(uint32_t* k, uint32_t* v, int64_t N, int n, cudaStream_t s);

@@ -66,3 +66,15 @@ def test_host_entry_point_long_arrays():
     h = torch.from_numpy(host.copy().view(np.float32)).pin_memory()
     gas.gas_sort_arrays_host(h)
     np.testing.assert_array_equal(h.numpy().view(np.uint32), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("onepass", ["0", "1"])
+@pytest.mark.parametrize("n", [16385, 32768, 32769, 65536])
+@pytest.mark.parametrize("dist", ["paper_uniform", "special_mix", "dup16"])
+def test_cluster_both_paths(monkeypatch, onepass, n, dist):
+    """Both f4 paths at every size: one pass (clusters of part-sized CTAs that
+    sort their parts) and two kernels (partition-only clusters, then the
+    variable-length classes over the 8 N parts)."""
+    monkeypatch.setenv("GAS_CLUSTER_ONEPASS", onepass)
+    host = datagen.fixed(dist, 9950 + n % 89, 0, max(3, 300_000 // n), n)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))

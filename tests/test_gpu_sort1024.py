@@ -212,3 +212,11 @@ def test_pipeline_small_batches_forced(monkeypatch, n, lead):
     for d in DISTS:  # homogeneous batches: each path leads once
         host = datagen.fixed(d, 9600 + n, 0, 64, n)
         np.testing.assert_array_equal(gpu_sort_fixed(host, lead=lead), oracle_sorted(host))
+
+
+@pytest.mark.parametrize("N", [1, 147, 148, 2959, 2960, 5000])
+@pytest.mark.parametrize("dist", ["paper_uniform", "spectra_intensity", "special_mix"])
+def test_fused_kernel_batch_sizes(N, dist):
+    """Batches below the pipeline threshold (16384 arrays) take the fused
+    kernel: fewer arrays than warps, than blocks, and several per warp."""
+    check(datagen.fixed(dist, 9990 + N, 0, N, 1000))
