@@ -39,6 +39,9 @@
 
 namespace gas {
 
+#ifndef GAS_ATOM_NOPRED  // shared atomics without predicates (see atoms_add4_if)
+#define GAS_ATOM_NOPRED 1
+#endif
 #ifndef GAS_BK_BLOCK
 #define GAS_BK_BLOCK 768  // one block of 24 warps per SM (80 registers): 4.22 ms; 20 warps as 640 / 320 / 160 / 128-thread blocks: 4.25 / 4.33 / 4.38 / 4.39 ms
 #endif
@@ -94,11 +97,23 @@ __device__ __forceinline__ float fmax_nan(float a, float b) {
 }
 // Shared-memory accesses as ordered (volatile) PTX; the predicated forms
 // compile to one predicated instruction instead of a branch.
-__device__ __forceinline__ uint32_t atoms_inc_if(bool p, uint32_t a) {
+__device__ __forceinline__ uint32_t atoms_inc_pred(bool p, uint32_t a) {
   uint32_t v = 0;
   asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %1, 0;\n\t@q atom.shared.add.u32 %0, [%2], 1;\n\t}"
                : "+r"(v) : "r"((uint32_t)p), "r"(a) : "memory");
   return v;
+}
+__device__ __forceinline__ uint32_t atoms_inc_if(bool p, uint32_t a) {  // see atoms_add4_if
+#if GAS_ATOM_NOPRED
+  uint32_t v;
+  asm volatile("atom.shared.add.u32 %0, [%1], %2;" : "=r"(v) : "r"(a), "r"(p ? 1u : 0u) : "memory");
+  return v;
+#else
+  uint32_t v = 0;
+  asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %1, 0;\n\t@q atom.shared.add.u32 %0, [%2], 1;\n\t}"
+               : "+r"(v) : "r"((uint32_t)p), "r"(a) : "memory");
+  return v;
+#endif
 }
 __device__ __forceinline__ uint32_t lds32(uint32_t a) {
   uint32_t v;
@@ -203,6 +218,26 @@ __device__ __forceinline__ void prefetch_l2(const uint32_t* p, int64_t words) {
 }
 
 
+// One lane (elect.sync: the lowest active lane) issues the bulk operation;
+// no branch, so no BSSY / BSYNC around it (GAS_BK_ELECT). The same lane always
+// wins while the warp is converged, which the bulk-group waits rely on.
+#ifndef GAS_BK_ELECT
+#define GAS_BK_ELECT 0
+#endif
+__device__ __forceinline__ void bulk_prefetch_elect(bool p, const void* g, uint32_t bytes) {
+  asm volatile("{\n\t.reg .pred e, q;\n\telect.sync _|e, 0xffffffff;\n\tsetp.ne.and.u32 q, %2, 0, e;\n\t"
+               "@q cp.async.bulk.prefetch.L2.global [%0], %1;\n\t}"
+               ::"l"(g), "r"(bytes), "r"((uint32_t)p) : "memory");
+}
+__device__ __forceinline__ void bulk_store_elect(void* g, uint32_t sa, uint32_t bytes) {
+  asm volatile("{\n\t.reg .pred e;\n\telect.sync _|e, 0xffffffff;\n\t"
+               "@e cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;\n\t@e cp.async.bulk.commit_group;\n\t}"
+               ::"l"(g), "r"(sa), "r"(bytes) : "memory");
+}
+__device__ __forceinline__ void bulk_wait_read_elect() {
+  asm volatile("{\n\t.reg .pred e;\n\telect.sync _|e, 0xffffffff;\n\t@e cp.async.bulk.wait_group.read 0;\n\t}" ::: "memory");
+}
+
 // Predicated forms of the global / shared accesses of the kernel below (one
 // predicated instruction each instead of a branch around it).
 __device__ __forceinline__ uint4 ldg_cs_if(bool p, const uint4* a) {
@@ -220,12 +255,31 @@ __device__ __forceinline__ void lds128_if(bool p, uint32_t a, uint32_t& x, uint3
   asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %4, 0;\n\t@q ld.shared.v4.u32 {%0, %1, %2, %3}, [%5];\n\t}"
                : "+r"(x), "+r"(y), "+r"(z), "+r"(w) : "r"((uint32_t)p), "r"(a) : "memory");
 }
-// Atomic add of 4 to the shared word at a, returning the old value (0 when !p).
-__device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
+// Atomic add of 4 to the shared word at a when p, returning the old value.
+// GAS_ATOM_NOPRED (default): the atomic always executes and adds 4 or 0 — ptxas
+// turns a predicated ATOMS into BSSY / BRA / ATOMS / BSYNC (3 extra
+// instructions per key whose predicate is not a constant); callers guarantee
+// that `a` is a valid counter address for every slot (slots past the end hold
+// a copy of a real key) and ignore the result when !p. atoms_add4_pred keeps
+// the predicated form (addresses that may be garbage when !p, and the kernels
+// where the unpredicated form measured slower: the key-linear kernel 4.50 ->
+// 4.57 ms, the split kernel's plain path on dup16 4.91 -> 4.95 ms; the value
+// kernel gained 4.096 -> 4.038 ms and the batch-CDF kernel 4.51 -> 4.44 ms,
+// profiles/r02_ab_atom_nopred.txt).
+__device__ __forceinline__ uint32_t atoms_add4_pred(bool p, uint32_t a) {
   uint32_t v = 0;
   asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %1, 0;\n\t@q atom.shared.add.u32 %0, [%2], 4;\n\t}"
                : "+r"(v) : "r"((uint32_t)p), "r"(a) : "memory");
   return v;
+}
+__device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
+#if GAS_ATOM_NOPRED
+  uint32_t v;
+  asm volatile("atom.shared.add.u32 %0, [%1], %2;" : "=r"(v) : "r"(a), "r"(p ? 4u : 0u) : "memory");
+  return v;
+#else
+  return atoms_add4_pred(p, a);
+#endif
 }
 
 // ---- Control block of the 512 < n <= 1024 pipeline (sort1024.cuh): device
@@ -390,12 +444,18 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
     }
 #if GAS_BK_PREFETCH
-    if (lane == 0 && a + GAS_BK_PREFETCH * nwarps < N)  // warm L2 with this warp's next array (one TMA bulk prefetch)
+    // warm L2 with this warp's next array (one TMA bulk prefetch)
+    if (GAS_BK_ELECT) {
+      bulk_prefetch_elect(a + GAS_BK_PREFETCH * nwarps < N, d + (a + GAS_BK_PREFETCH * nwarps) * (int64_t)n, (uint32_t)n * 4u);
+    } else if (lane == 0 && a + GAS_BK_PREFETCH * nwarps < N) {
       asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + (a + GAS_BK_PREFETCH * nwarps) * (int64_t)n),
                    "r"((uint32_t)n * 4u) : "memory");
+    }
 #endif
 #if GAS_BK_TMA_STORE
-    if (lane == 0) asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory");  // the previous bulk store has read the staging
+    // the previous bulk store has read the staging (the lane that issued it waits)
+    if (GAS_BK_ELECT) bulk_wait_read_elect();
+    else if (lane == 0) asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory");
     __syncwarp();
 #endif
     // slots past the end repeat k[0] so that min / max need no predicates
@@ -488,7 +548,7 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
             uint32_t sa[GAS_BK_GROUP];
 #pragma unroll
             for (int r = g; r < g + GAS_BK_GROUP; ++r)
-              sa[r - g] = atoms_add4_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, __umulhi(k[r] - klo, mk) * 4u + cnt_sa);
+              sa[r - g] = atoms_add4_pred((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, __umulhi(k[r] - klo, mk) * 4u + cnt_sa);
 #pragma unroll
             for (int r = g; r < g + GAS_BK_GROUP; ++r)
               sts32_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, min(sa[r - g], slot_last), k[r]);
@@ -500,7 +560,7 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
 #pragma unroll
             for (int r = g; r < g + GAS_BK_GROUP; ++r) {
               kk[r - g] = key_from_bits(k[r]);
-              sa[r - g] = atoms_add4_if((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, __umulhi(kk[r - g] - klo, mk) * 4u + cnt_sa);
+              sa[r - g] = atoms_add4_pred((r >> 2) < 4 || lane + 32 * (r >> 2) < nc, __umulhi(kk[r - g] - klo, mk) * 4u + cnt_sa);
             }
 #pragma unroll
             for (int r = g; r < g + GAS_BK_GROUP; ++r)
@@ -578,7 +638,9 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
       if (raw) {  // the staged array is contiguous: one TMA bulk store (the copy engine reads shared memory)
         asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
         __syncwarp();
-        if (lane == 0) {
+        if (GAS_BK_ELECT) {
+          bulk_store_elect(dst, stage_sa, (uint32_t)n * 4u);
+        } else if (lane == 0) {
           asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;"
                        ::"l"(dst), "r"(stage_sa), "r"((uint32_t)n * 4u) : "memory");
           asm volatile("cp.async.bulk.commit_group;" ::: "memory");

@@ -269,7 +269,7 @@ static __global__ void __launch_bounds__(kBk2Block, 1)
         uint32_t sa[4];
 #pragma unroll
         for (int r = g; r < g + 4; ++r)
-          sa[r - g] = atoms_add4_if(live && ((r >> 2) < 2 || hl + 16 * (r >> 2) < nc), bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
+          sa[r - g] = atoms_add4_pred(live && ((r >> 2) < 2 || hl + 16 * (r >> 2) < nc), bucket_bits(k[r], vmin, s) * 4u + cnt_b0);
 #pragma unroll
         for (int r = g; r < g + 4; ++r)
           sts32_if(live && ((r >> 2) < 2 || hl + 16 * (r >> 2) < nc), min(sa[r - g], slot_last), raw ? k[r] : key_from_bits(k[r]));

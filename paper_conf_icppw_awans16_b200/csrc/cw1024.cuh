@@ -82,15 +82,26 @@ constexpr int kCwSmemBytes = (kCwBlock / 32) * kCwWarpBytes;
 // conflict-free.
 __device__ __forceinline__ uint32_t cw_swz(uint32_t w) { return w ^ ((w >> 3) & 0x1Cu); }
 
+// (GAS_ATOM_NOPRED: unpredicated, adding 0 when !p; see atoms_add4_if in bucket1024.cuh)
 __device__ __forceinline__ void reds_add_if(bool p, uint32_t a, uint32_t v) {
+#if GAS_ATOM_NOPRED
+  asm volatile("red.shared.add.u32 [%0], %1;" ::"r"(a), "r"(p ? v : 0u) : "memory");
+#else
   asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %0, 0;\n\t@q red.shared.add.u32 [%1], %2;\n\t}"
                ::"r"((uint32_t)p), "r"(a), "r"(v) : "memory");
+#endif
 }
 __device__ __forceinline__ uint32_t atoms_add_if(bool p, uint32_t a, uint32_t v) {
+#if GAS_ATOM_NOPRED
+  uint32_t r;
+  asm volatile("atom.shared.add.u32 %0, [%1], %2;" : "=r"(r) : "r"(a), "r"(p ? v : 0u) : "memory");
+  return r;
+#else
   uint32_t r = 0;
   asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %1, 0;\n\t@q atom.shared.add.u32 %0, [%2], %3;\n\t}"
                : "+r"(r) : "r"((uint32_t)p), "r"(a), "r"(v) : "memory");
   return r;
+#endif
 }
 
 __device__ __forceinline__ uint32_t cw_kl_shift(uint32_t kmin, uint32_t kmax) {

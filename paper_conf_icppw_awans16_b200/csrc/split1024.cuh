@@ -99,7 +99,8 @@ __device__ __forceinline__ bool sp_scatter(const uint32_t (&k)[32], int lane, in
 #pragma unroll
     for (int r = g; r < g + 4; ++r) {
       row[r - g] = SP ? sp_row(k[r], m) : pl_row(k[r], vmin, s);
-      c[r - g] = atoms_inc_if(cw_valid<VEC>(r, lane, n), cnt_sa + row[r - g] * 4);
+      c[r - g] = SP ? atoms_inc_if(cw_valid<VEC>(r, lane, n), cnt_sa + row[r - g] * 4)
+                    : atoms_inc_pred(cw_valid<VEC>(r, lane, n), cnt_sa + row[r - g] * 4);
     }
     uint32_t ra[4], kk[4];
     bool ov[4];
