@@ -122,7 +122,7 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
   const uint32_t row1 = row0 + T * (kBkRowWords * 4);
   const int nc = n >> 2;
   const int head = TMA ? (int)((reinterpret_cast<uintptr_t>(arr) >> 2) & 3u) : 0;  // staging shift (0 when VEC)
-  if (TMA && t == 0) asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory");  // ordered by the first barrier
+  if (TMA && warp == 0) bulk_wait_read_elect();  // thread 0 (the issuing lane); ordered by the first barrier
   // key r of this thread: VEC element 4 (t + T (r/4)) + r%4, else element t + T r
   auto valid = [&](int r) -> bool {
     if (VEC) return (r >> 2) < 4 || t + T * (r >> 2) < nc;
@@ -299,12 +299,8 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
       asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // this thread's staging writes -> async proxy
       bar_cta<WR>(bar);
       const int h0 = (4 - head) & 3, h1 = h0 + ((n - h0) & ~3);  // [h0, h1): 16-byte aligned in both memories
-      if (t == 0 && h1 > h0) {
-        asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;"
-                     ::"l"(arr + h0), "r"(stage_sa + (uint32_t)(head + h0) * 4u), "r"((uint32_t)(h1 - h0) * 4u)
-                     : "memory");
-        asm volatile("cp.async.bulk.commit_group;" ::: "memory");
-      }
+      if (warp == 0 && h1 > h0)  // one elected lane of warp 0 (thread 0, which also waits for it)
+        bulk_store_elect(arr + h0, stage_sa + (uint32_t)(head + h0) * 4u, (uint32_t)(h1 - h0) * 4u);
       if (t < h0) st_stream(arr + t, lds32(stage_sa + (head + t) * 4));
       else if (t >= 4 && t - 4 + h1 < n) st_stream(arr + (t - 4 + h1), lds32(stage_sa + (head + t - 4 + h1) * 4));
     } else {
@@ -377,7 +373,7 @@ __global__ void __launch_bounds__(bkc_block<WR>(), bkc_launch_min_blocks<WR>())
   const int64_t stride = (int64_t)gridDim.x * GR;
   for (int64_t a = (int64_t)blockIdx.x * GR + grp; a < N; a += stride) {
 #if GAS_BKC_PREFETCH
-    if (t == 0 && a + stride < N) prefetch_l2(d + (a + stride) * (int64_t)n, n);
+    if (t < 32) prefetch_l2_elect(a + stride < N, d + (a + stride) * (int64_t)n, n);
 #endif
     bucket_sort_cta<W, WR, VEC>(d + a * (int64_t)n, n, sm, one, t, bar);
   }
@@ -421,7 +417,7 @@ __global__ void __launch_bounds__(32 * WR, bkc_min_blocks<WR>())
         const int nx = __ffs(mask) - 1;
         const int64_t nlo = __shfl_sync(0xffffffffu, my_lo, nx);
         const int64_t nlen = __shfl_sync(0xffffffffu, my_len, nx);
-        if (t == 0) prefetch_l2(d + nlo, nlen);
+        if (t < 32) prefetch_l2_elect(true, d + nlo, nlen);
       }
 #endif
       bucket_sort_cta<W, WR, false, RV>(d + lo, len, sm, one, t, bar);

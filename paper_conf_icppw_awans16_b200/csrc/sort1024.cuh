@@ -475,7 +475,7 @@ __global__ void __launch_bounds__(kCwBlock, 1) k_s1_count(uint32_t* __restrict__
     uint32_t k[32];
     s1_load<VEC>(k, arr, n, lane);
 #if GAS_BK_PREFETCH
-    if (lane == 0 && a + nwarps < N) prefetch_l2(d + (a + nwarps) * (int64_t)n, n);
+    prefetch_l2_elect(a + nwarps < N, d + (a + nwarps) * (int64_t)n, n);
 #endif
     uint32_t umin = k[0], umax = k[0];
 #pragma unroll

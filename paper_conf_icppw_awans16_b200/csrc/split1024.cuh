@@ -184,7 +184,7 @@ __global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__
     uint32_t k[32];
     s1_load<VEC>(k, arr, n, lane);
 #if GAS_BK_PREFETCH
-    if (flag == kS1Split && lane == 0 && i + nwarps < count) prefetch_l2(d + (i + nwarps) * (int64_t)n, n);
+    prefetch_l2_elect(flag == kS1Split && i + nwarps < count, d + (i + nwarps) * (int64_t)n, n);
 #endif
     // ---- key range: NaN / inf present? min / max of the normal values (SP) or of all keys (plain)
     uint32_t kmin = 0xFFFFFFFFu, kmax = 0u;

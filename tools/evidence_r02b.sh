@@ -13,11 +13,9 @@ done
 timeout 900 python bench.py --config 3 --cpu-seconds 60 --steps 10 > gpurun_out/e_c3.json 2> gpurun_out/e_c3.err
 timeout 600 python bench.py --variant pairs --no-e2e --steps 10 > gpurun_out/e_pairs.json 2> gpurun_out/e_pairs.err
 timeout 600 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/e_launches.csv python bench.py --steps 3 --warmup 2 --no-e2e --no-cpu-baseline > /dev/null 2>&1
-timeout 900 ncu --set full --clock-control none --import-source on -k regex:k_fixed_bucket1024 -s 2 -c 1 -o gpurun_out/e_ncu_bk python bench.py --steps 2 --warmup 1 --no-e2e --no-cpu-baseline > gpurun_out/e_ncu_bk.log 2>&1
-for tool in memcheck racecheck synccheck; do
-  timeout 1500 compute-sanitizer --tool $tool --print-limit 20 --error-exitcode 9 python tools/sanitize_cases_r02.py > gpurun_out/e_sanitize_$tool.log 2>&1
-  echo "$tool rc=$?" >> gpurun_out/e_sanitize_summary.txt; tail -2 gpurun_out/e_sanitize_$tool.log >> gpurun_out/e_sanitize_summary.txt
-done
+timeout 900 ncu --set full --clock-control none --import-source on --kernel-name-base mangled -k regex:_ZN3gas18k_fixed_bucket1024ILb1ELi0E -s 1 -c 1 -o gpurun_out/e_ncu_bk0 python bench.py --steps 2 --warmup 1 --no-e2e --no-cpu-baseline > gpurun_out/e_ncu_bk0.log 2>&1
+timeout 900 ncu --set full --clock-control none --import-source on --kernel-name-base mangled -k regex:_ZN3gas18k_fixed_bucket1024ILb1ELi2E -s 1 -c 1 -o gpurun_out/e_ncu_cdf python bench.py --steps 2 --warmup 1 --no-e2e --no-cpu-baseline --dist spectra_intensity > gpurun_out/e_ncu_cdf.log 2>&1
+# (compute-sanitizer is closed on this pool: profiles/r02_compute_sanitizer_closed.txt)
 tail -2 gpurun_out/e_smoke.log; tail -2 gpurun_out/e_pytest_gpu.log; cut -c1-300 gpurun_out/e_bench.json
 python - <<'PY'
 import json
@@ -30,4 +28,3 @@ for f in ('gpurun_out/e_c3.json', 'gpurun_out/e_pairs.json'):
         print(f, round(d['ms_per_step'], 3), round(d['roofline']['frac'], 4), c.get('sample'), c.get('gpu_bit_exact_on_sample'), (d.get('e2e') or {}).get('ms_per_step'))
     except Exception as e: print(f, 'ERR', e)
 PY
-cat gpurun_out/e_sanitize_summary.txt
