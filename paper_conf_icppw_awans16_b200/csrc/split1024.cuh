@@ -41,6 +41,9 @@
 
 namespace gas {
 
+#ifndef GAS_SP_TMA  // 16-byte rows: stage float bits and leave through one TMA bulk store per array
+#define GAS_SP_TMA 1   // measured: dup16 4.88 -> 4.61 ms, special_mix 6.98 -> 7.11 (only for plain arrays: special_mix 7.69)
+#endif
 constexpr int kSpBlock = 768;                       // 24 warps per SM (as the bucket kernel)
 constexpr int kSpCntWords = 68;                     // 64 row counters + 4 run counters (-inf, -0, +0, +inf)
 constexpr int kSpCntBytes = kSpCntWords * 4;
@@ -183,6 +186,11 @@ __global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__
     uint32_t* const arr = d + a * (int64_t)n;
     uint32_t k[32];
     s1_load<VEC>(k, arr, n, lane);
+    constexpr bool TB = VEC && GAS_SP_TMA;  // stage bits, bulk store
+    if constexpr (TB) {
+      bulk_wait_read_elect();  // the previous array's bulk store has read the staging rows
+      __syncwarp();
+    }
 #if GAS_BK_PREFETCH
     prefetch_l2_elect(flag == kS1Split && i + nwarps < count, d + (i + nwarps) * (int64_t)n, n);
 #endif
@@ -322,15 +330,15 @@ __global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__
         if (__any_sync(0xffffffffu, keys)) {  // else every row of this round is empty or a run
           if (__any_sync(0xffffffffu, keys && tb >= 2u)) sortn_bk<32>(k, one);
 #pragma unroll
-          for (int q = 0; q < 32; ++q) sts32_if(keys && (uint32_t)q < tb, ob + q * 4, k[q]);
+          for (int q = 0; q < 32; ++q) sts32_if(keys && (uint32_t)q < tb, ob + q * 4, TB ? bits_from_key(k[q]) : k[q]);
         }
       }
     }
     if (!bad) {
       // ---- runs: equal-key overflow rows, then (SP) -inf, -0, +0, +inf
       // each lane writes its own overflow rows' runs; runs longer than 256 keys are written by the warp
-      if (t1 > 32u && t1 <= 256u) sp_fill(stage_sa, base1, t1, rep1);
-      if (t0 > 32u && t0 <= 256u) sp_fill(stage_sa, base0, t0, rep0);
+      if (t1 > 32u && t1 <= 256u) sp_fill(stage_sa, base1, t1, TB ? bits_from_key(rep1) : rep1);
+      if (t0 > 32u && t0 <= 256u) sp_fill(stage_sa, base0, t0, TB ? bits_from_key(rep0) : rep0);
       uint32_t om0 = __ballot_sync(0xffffffffu, t0 > 256u), om1 = __ballot_sync(0xffffffffu, t1 > 256u);
       while (om0 | om1) {
         const bool hi = om0 == 0u;
@@ -339,21 +347,27 @@ __global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__
         else om0 &= om0 - 1u;
         const uint32_t st = __shfl_sync(0xffffffffu, hi ? base1 : base0, owner);
         const uint32_t len = __shfl_sync(0xffffffffu, hi ? t1 : t0, owner);
-        const uint32_t val = __shfl_sync(0xffffffffu, hi ? rep1 : rep0, owner);
+        const uint32_t vk = __shfl_sync(0xffffffffu, hi ? rep1 : rep0, owner);
+        const uint32_t val = TB ? bits_from_key(vk) : vk;
         for (uint32_t p = lane; p < len; p += 32) sts32(stage_sa + (st + p) * 4, val);
       }
       if (sp) {
         const uint32_t s_ninf = __shfl_sync(0xffffffffu, base0 + t0, 1);
         const uint32_t zs = __shfl_sync(0xffffffffu, zrow < 32u ? base0 + t0 : base1 + t1, (int)(zrow & 31u));
         const uint32_t s_pinf = __shfl_sync(0xffffffffu, base1, 30);
-        for (uint32_t p = lane; p < r_ninf; p += 32) sts32(stage_sa + (s_ninf + p) * 4, 0x007FFFFFu);
-        for (uint32_t p = lane; p < r_nz; p += 32) sts32(stage_sa + (zs + p) * 4, 0x7FFFFFFFu);
-        for (uint32_t p = lane; p < r_pz; p += 32) sts32(stage_sa + (zs + r_nz + p) * 4, 0x80000000u);
-        for (uint32_t p = lane; p < r_pinf; p += 32) sts32(stage_sa + (s_pinf + p) * 4, 0xFF800000u);
+        // keys of -inf, -0, +0, +inf (TB: their bit patterns)
+        for (uint32_t p = lane; p < r_ninf; p += 32) sts32(stage_sa + (s_ninf + p) * 4, TB ? 0xFF800000u : 0x007FFFFFu);
+        for (uint32_t p = lane; p < r_nz; p += 32) sts32(stage_sa + (zs + p) * 4, TB ? 0x80000000u : 0x7FFFFFFFu);
+        for (uint32_t p = lane; p < r_pz; p += 32) sts32(stage_sa + (zs + r_nz + p) * 4, TB ? 0x00000000u : 0x80000000u);
+        for (uint32_t p = lane; p < r_pinf; p += 32) sts32(stage_sa + (s_pinf + p) * 4, TB ? 0x7F800000u : 0xFF800000u);
       }
       __syncwarp();
       // ---- store in place (keys -> bits)
-      if constexpr (VEC) {
+      if constexpr (TB) {
+        asm volatile("fence.proxy.async.shared::cta;" ::: "memory");  // staging writes -> async proxy
+        __syncwarp();
+        bulk_store_elect(arr, stage_sa, (uint32_t)n * 4u);
+      } else if constexpr (VEC) {
         uint4* const dst = reinterpret_cast<uint4*>(arr);
         const int nc = n >> 2;
 #pragma unroll
@@ -379,6 +393,7 @@ __global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__
     }
     __syncwarp();
   }
+  if (VEC && GAS_SP_TMA) asm volatile("{\n\t.reg .pred e;\n\telect.sync _|e, 0xffffffff;\n\t@e cp.async.bulk.wait_group 0;\n\t}" ::: "memory");  // bulk stores complete before exit
 }
 
 }  // namespace gas
