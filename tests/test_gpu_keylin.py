@@ -167,3 +167,14 @@ def test_natural_routing_spectra_intensity(monkeypatch):
     before = gas.launch_count()
     check(host)
     assert gas.launch_count() - before == 6
+
+
+@pytest.mark.parametrize("sigma", [1.0, 2.0, 3.0, 4.0])
+def test_natural_routing_lognormal(monkeypatch, sigma):
+    """Unforced pipeline on log-normal batches (spectra-like intensities,
+    mu = 8, sigma = 1..4): whichever path the sampler picks (value buckets,
+    batch-CDF buckets, counting sort), every array bit-exact."""
+    monkeypatch.delenv("GAS_S1_FORCE", raising=False)
+    rng = np.random.default_rng(int(sigma * 100))
+    host = np.asarray(rng.lognormal(8.0, sigma, size=(20000, 1000)), dtype=np.float32).view(np.uint32)
+    check(np.ascontiguousarray(host))
