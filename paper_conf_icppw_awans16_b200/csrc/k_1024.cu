@@ -18,7 +18,7 @@ cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   constexpr int smem = gas::warp_smem_bytes<KPT, G>();
   constexpr int arrays_per_block = (blk / 32) * (32 / G);
   auto k = gas::k_fixed_warp<KPT, G, VEC>;
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  const cudaError_t e = set_smem_cached(reinterpret_cast<const void*>(k), smem);
   if (e != cudaSuccess) return e;
   const int grid = persistent_grid_smem(k, blk, smem, (N + arrays_per_block - 1) / arrays_per_block);
   k<<<grid, blk, smem, s>>>(d, N, n, 1u);
@@ -29,8 +29,7 @@ cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
 
 cudaError_t launch_fixed_1024_tma(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   // per-device attribute: set on every call (cheap), the current device may change
-  const cudaError_t attr = cudaFuncSetAttribute(gas::k_fixed_1024_tma, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                                gas::kTmaSmemBytes);
+  const cudaError_t attr = set_smem_cached(reinterpret_cast<const void*>(gas::k_fixed_1024_tma), gas::kTmaSmemBytes);
   if (attr != cudaSuccess) return attr;
   int per_sm = 0;
   if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, gas::k_fixed_1024_tma, gas::kWarpBlock,
@@ -48,7 +47,7 @@ cudaError_t launch_fixed_1024_tma(uint32_t* d, int64_t N, int n, cudaStream_t s)
 template <bool VEC>
 cudaError_t launch_fixed_bucket1024(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   auto k = VEC ? gas::k_fixed_bucket1024<false> : gas::k_fixed_bucket1024_any<false, false>;
-  const cudaError_t attr = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kBkSmemBytes);
+  const cudaError_t attr = set_smem_cached(reinterpret_cast<const void*>(k), gas::kBkSmemBytes);
   if (attr != cudaSuccess) return attr;
   const int grid = persistent_grid_smem(k, gas::kBkBlock, gas::kBkSmemBytes,
                                         (N + gas::kBkBlock / 32 - 1) / (gas::kBkBlock / 32));
@@ -62,7 +61,7 @@ cudaError_t launch_fixed_bucket1024(uint32_t* d, int64_t N, int n, cudaStream_t 
 template <bool VEC>
 cudaError_t launch_fixed_sort1024(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   auto k = gas::k_fixed_sort1024<VEC>;
-  const cudaError_t attr = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kS1SmemBytes);
+  const cudaError_t attr = set_smem_cached(reinterpret_cast<const void*>(k), gas::kS1SmemBytes);
   if (attr != cudaSuccess) return attr;
   const int grid = persistent_grid_smem(k, gas::kS1Block, gas::kS1SmemBytes,
                                         (N + gas::kS1Block / 32 - 1) / (gas::kS1Block / 32));
@@ -88,7 +87,7 @@ cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   e = cudaGetLastError();
   if (e == cudaSuccess) {
     auto k = VEC ? gas::k_fixed_bucket1024<true> : gas::k_fixed_bucket1024_any<false, true>;
-    e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kBkSmemBytes);
+    e = set_smem_cached(reinterpret_cast<const void*>(k), gas::kBkSmemBytes);
     if (e == cudaSuccess) {
       const int grid = persistent_grid_smem(k, gas::kBkBlock, gas::kBkSmemBytes,
                                             (N + gas::kBkBlock / 32 - 1) / (gas::kBkBlock / 32));
@@ -101,7 +100,7 @@ cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
     auto k = map == gas::kMapKeyLin ? gas::k_fixed_bucket1024<true, gas::kMapKeyLin>
                                     : gas::k_fixed_bucket1024<true, gas::kMapCdf>;
     const int smem = gas::kBkSmemBytes + (map == gas::kMapCdf ? gas::kCdfEntries * 8 : 0);
-    e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+    e = set_smem_cached(reinterpret_cast<const void*>(k), smem);
     if (e == cudaSuccess) {
       const int grid = persistent_grid_smem(k, gas::kBkBlock, smem, (N + gas::kBkBlock / 32 - 1) / (gas::kBkBlock / 32));
       k<<<grid, gas::kBkBlock, smem, s>>>(d, N, n, 1u, ctl);
@@ -110,7 +109,7 @@ cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   }
   if (e == cudaSuccess) {
     auto k = gas::k_s1_count<VEC>;
-    e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kCwSmemBytes);
+    e = set_smem_cached(reinterpret_cast<const void*>(k), gas::kCwSmemBytes);
     if (e == cudaSuccess) {
       const int grid = persistent_grid_smem(k, gas::kCwBlock, gas::kCwSmemBytes,
                                             (N + gas::kCwBlock / 32 - 1) / (gas::kCwBlock / 32));
@@ -120,7 +119,7 @@ cudaError_t launch_s1_pipeline(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   }
   if (e == cudaSuccess) {
     auto k = gas::k_s1_split<VEC>;
-    e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kSpSmemBytes);
+    e = set_smem_cached(reinterpret_cast<const void*>(k), gas::kSpSmemBytes);
     if (e == cudaSuccess) {
       const int grid = persistent_grid_smem(k, gas::kSpBlock, gas::kSpSmemBytes,
                                             (N + gas::kSpBlock / 32 - 1) / (gas::kSpBlock / 32));

@@ -19,7 +19,7 @@ cudaError_t launch_cluster(uint32_t* d, int64_t N, int n, uint32_t* fail, int64_
   using G = gas::ClCfg<W, WR, C, MAXN>;
   auto k = gas::k_cluster_sort<W, WR, C, MAXN, PART>;
   constexpr int smem = PART ? 0 : G::SMEM;
-  cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  cudaError_t e = set_smem_cached(reinterpret_cast<const void*>(k), smem);
   if (e == cudaSuccess && C > 8) e = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
   if (e != cudaSuccess) return e;
   cudaLaunchAttribute attr[1];

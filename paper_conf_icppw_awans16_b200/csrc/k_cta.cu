@@ -13,7 +13,7 @@ template <int W, int WR, bool VEC>
 cudaError_t launch_fixed_cta(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   auto k = gas::k_fixed_cta<W, WR, VEC>;
   constexpr int smem = gas::cta_smem_bytes<W, WR>();
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  const cudaError_t e = set_smem_cached(reinterpret_cast<const void*>(k), smem);
   if (e != cudaSuccess) return e;
   k<<<persistent_grid_smem(k, 32 * WR, smem, N), 32 * WR, smem, s>>>(d, N, n, 1u);
   return cudaGetLastError();
@@ -26,7 +26,7 @@ cudaError_t launch_fixed_bucket_cta(uint32_t* d, int64_t N, int n, cudaStream_t 
   auto k = gas::k_fixed_bucket_cta<W, WR, VEC>;
   constexpr int gr = gas::bkc_groups<WR>(), blk = gas::bkc_block<WR>();
   constexpr int smem = gas::BkCta<W, WR>::SMEM * gr;
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  const cudaError_t e = set_smem_cached(reinterpret_cast<const void*>(k), smem);
   if (e != cudaSuccess) return e;
   k<<<persistent_grid_smem(k, blk, smem, (N + gr - 1) / gr), blk, smem, s>>>(d, N, n, 1u);
   return cudaGetLastError();

@@ -15,7 +15,7 @@ cudaError_t launch_offsets_bucket(uint32_t* d, const int64_t* off, int64_t N, in
   auto k = gas::k_offsets_bucket<W, WR, RV>;
   constexpr int gr = 1, blk = 32 * WR;
   constexpr int smem = gas::BkCta<W, WR>::SMEM * gr;
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  const cudaError_t e = set_smem_cached(reinterpret_cast<const void*>(k), smem);
   if (e != cudaSuccess) return e;
   k<<<persistent_grid_smem(k, blk, smem, ((N + 31) / 32 + gr - 1) / gr), blk, smem, s>>>(d, off, N, lo, hi, ctr, 1u);
   return cudaGetLastError();
@@ -27,7 +27,7 @@ cudaError_t launch_offsets_warp(uint32_t* d, const int64_t* off, int64_t N, cuda
   constexpr int blk = gas::warp_block<G>();
   constexpr int smem = gas::warp_smem_bytes<KPT, G>();
   auto k = gas::k_offsets_warp<KPT, G>;
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  const cudaError_t e = set_smem_cached(reinterpret_cast<const void*>(k), smem);
   if (e != cudaSuccess) return e;
   const int64_t windows = (N + 31) / 32;
   const int grid = persistent_grid_smem(k, blk, smem, (windows + blk / 32 - 1) / (blk / 32));
@@ -40,7 +40,7 @@ cudaError_t launch_offsets_cta(uint32_t* d, const int64_t* off, int64_t N, int64
                                unsigned long long* ctr, cudaStream_t s) {
   auto k = gas::k_offsets_cta<W, WR>;
   constexpr int smem = gas::cta_smem_bytes<W, WR>();
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  const cudaError_t e = set_smem_cached(reinterpret_cast<const void*>(k), smem);
   if (e != cudaSuccess) return e;
   k<<<persistent_grid_smem(k, 32 * WR, smem, (N + 31) / 32), 32 * WR, smem, s>>>(d, off, N, lo, hi, ctr, 1u);
   return cudaGetLastError();

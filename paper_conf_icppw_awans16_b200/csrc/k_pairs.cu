@@ -13,7 +13,7 @@ template <int KPT, int G, int W>
 cudaError_t launch_pairs(uint32_t* k, uint32_t* v, int64_t N, int n, cudaStream_t s, const uint32_t* list = nullptr) {
   using C = gas::PairsCfg<KPT, G, W>;
   auto kern = gas::k_pairs<KPT, G, W>;
-  cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, C::SMEM);
+  cudaError_t e = set_smem_cached(reinterpret_cast<const void*>(kern), C::SMEM);
   if (e != cudaSuccess) return e;
   int per_sm = 0;
   if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, C::TPB, C::SMEM) != cudaSuccess || per_sm <= 0)
@@ -34,7 +34,7 @@ cudaError_t launch_pairs_bucket1024(uint32_t* k, uint32_t* v, int64_t N, int n, 
   uint32_t* fail = static_cast<uint32_t*>(ws);
   e = cudaMemsetAsync(fail, 0, 4, s);
   if (e == cudaSuccess)
-    e = cudaFuncSetAttribute(gas::k_pairs_bucket1024, cudaFuncAttributeMaxDynamicSharedMemorySize, gas::kPbSmemBytes);
+    e = set_smem_cached(reinterpret_cast<const void*>(gas::k_pairs_bucket1024), gas::kPbSmemBytes);
   if (e == cudaSuccess) {
     const int grid = persistent_grid_smem(gas::k_pairs_bucket1024, gas::kPbBlock, gas::kPbSmemBytes,
                                           (N + gas::kPbBlock / 32 - 1) / (gas::kPbBlock / 32));

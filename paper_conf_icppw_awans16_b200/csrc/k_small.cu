@@ -15,7 +15,7 @@ cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
   constexpr int smem = gas::warp_smem_bytes<KPT, G>();
   constexpr int arrays_per_block = (blk / 32) * (32 / G);
   auto k = gas::k_fixed_warp<KPT, G, VEC>;
-  const cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  const cudaError_t e = set_smem_cached(reinterpret_cast<const void*>(k), smem);
   if (e != cudaSuccess) return e;
   const int grid = persistent_grid_smem(k, blk, smem, (N + arrays_per_block - 1) / arrays_per_block);
   k<<<grid, blk, smem, s>>>(d, N, n, 1u);
@@ -26,8 +26,7 @@ cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
 
 // Bucket-then-network kernel for 256 < n <= 512 with aligned rows (bucket512.cuh).
 cudaError_t launch_fixed_bucket512(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  const cudaError_t attr = cudaFuncSetAttribute(gas::k_fixed_bucket512, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                                gas::kBk5SmemBytes);
+  const cudaError_t attr = set_smem_cached(reinterpret_cast<const void*>(gas::k_fixed_bucket512), gas::kBk5SmemBytes);
   if (attr != cudaSuccess) return attr;
   const int grid = persistent_grid_smem(gas::k_fixed_bucket512, gas::kBk5Block, gas::kBk5SmemBytes,
                                         (N + GAS_BK5_WARPS - 1) / GAS_BK5_WARPS);
@@ -38,8 +37,7 @@ cudaError_t launch_fixed_bucket512(uint32_t* d, int64_t N, int n, cudaStream_t s
 
 // Bucket-then-network kernel for 128 < n <= 256 with aligned rows (bucket512.cuh, half a warp per array).
 cudaError_t launch_fixed_bucket256(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  const cudaError_t attr = cudaFuncSetAttribute(gas::k_fixed_bucket256, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                                gas::kBk2SmemBytes);
+  const cudaError_t attr = set_smem_cached(reinterpret_cast<const void*>(gas::k_fixed_bucket256), gas::kBk2SmemBytes);
   if (attr != cudaSuccess) return attr;
   const int grid = persistent_grid_smem(gas::k_fixed_bucket256, gas::kBk2Block, gas::kBk2SmemBytes,
                                         (N + 2 * GAS_BK2_WARPS - 1) / (2 * GAS_BK2_WARPS));

@@ -12,11 +12,58 @@
 
 namespace gas_host {
 
+// Host-side launch bookkeeping is cached (per device, per kernel): a call on a
+// small batch is otherwise dominated by driver queries made before its first
+// launch (the GPU idles meanwhile).
+constexpr int kLaunchCacheDevices = 64;
+inline int current_device() {
+  int dev = 0;
+  if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= kLaunchCacheDevices) dev = 0;
+  return dev;
+}
 inline int num_sms() {
-  int dev = 0, sms = 0;
-  if (cudaGetDevice(&dev) != cudaSuccess) return 148;
+  static std::atomic<int> cache[kLaunchCacheDevices];  // 0 = not queried yet
+  const int dev = current_device();
+  int sms = cache[dev].load(std::memory_order_relaxed);
+  if (sms > 0) return sms;
   if (cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev) != cudaSuccess || sms <= 0) return 148;
+  cache[dev].store(sms, std::memory_order_relaxed);
   return sms;
+}
+// Resident blocks per SM of (kernel, threads, dynamic shared memory) on the current device, cached.
+inline int occupancy_cached(const void* kernel, int threads, int smem) {
+  struct Entry { const void* k; int threads, smem, dev, per_sm; };
+  static std::mutex mu;
+  static Entry tab[256];
+  static int used = 0;
+  const int dev = current_device();
+  {
+    std::lock_guard<std::mutex> lock(mu);
+    for (int i = 0; i < used; ++i)
+      if (tab[i].k == kernel && tab[i].threads == threads && tab[i].smem == smem && tab[i].dev == dev) return tab[i].per_sm;
+  }
+  int per_sm = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kernel, threads, smem) != cudaSuccess || per_sm <= 0) {
+    (void)cudaGetLastError();
+    return 1;  // not cached: a failed query is retried next time
+  }
+  std::lock_guard<std::mutex> lock(mu);
+  if (used < 256) tab[used++] = Entry{kernel, threads, smem, dev, per_sm};
+  return per_sm;
+}
+// cudaFuncSetAttribute(MaxDynamicSharedMemorySize) once per (kernel, device, size).
+inline cudaError_t set_smem_cached(const void* kernel, int smem) {
+  struct Entry { const void* k; int smem, dev; };
+  static std::mutex mu;
+  static Entry tab[256];
+  static int used = 0;
+  const int dev = current_device();
+  std::lock_guard<std::mutex> lock(mu);
+  for (int i = 0; i < used; ++i)
+    if (tab[i].k == kernel && tab[i].smem == smem && tab[i].dev == dev) return cudaSuccess;
+  const cudaError_t e = cudaFuncSetAttribute(kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+  if (e == cudaSuccess && used < 256) tab[used++] = Entry{kernel, smem, dev};
+  return e;
 }
 
 inline int32_t size_class(int64_t n) {  // smallest power of two >= n, n >= 2
@@ -39,9 +86,7 @@ inline int64_t grid_cap() {
 
 template <typename K>
 inline int persistent_grid(K kernel, int threads, int64_t blocks_needed) {
-  int per_sm = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kernel, threads, 0) != cudaSuccess || per_sm <= 0)
-    per_sm = 1;
+  const int per_sm = occupancy_cached(reinterpret_cast<const void*>(kernel), threads, 0);
   int64_t cap = (int64_t)per_sm * num_sms();
   if (grid_cap() > 0 && grid_cap() < cap) cap = grid_cap();
   return (int)(blocks_needed < cap ? (blocks_needed > 0 ? blocks_needed : 1) : cap);
@@ -49,9 +94,7 @@ inline int persistent_grid(K kernel, int threads, int64_t blocks_needed) {
 
 template <typename K>
 inline int persistent_grid_smem(K kernel, int threads, int smem, int64_t blocks_needed) {
-  int per_sm = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kernel, threads, smem) != cudaSuccess || per_sm <= 0)
-    per_sm = 1;
+  const int per_sm = occupancy_cached(reinterpret_cast<const void*>(kernel), threads, smem);
   int64_t cap = (int64_t)per_sm * num_sms();
   if (grid_cap() > 0 && grid_cap() < cap) cap = grid_cap();
   return (int)(blocks_needed < cap ? (blocks_needed > 0 ? blocks_needed : 1) : cap);
