@@ -504,7 +504,7 @@ def main():
                          "peak_source": peak_src, "kernel": kernel_hint,
                          "algorithmic_bytes_per_launch": alg_bytes,
                          "timed": "the whole C-ABI call per step (CUDA events on its stream); for 512 < n <= 1024 "
-                                  "and N >= 16384 that is the sort1024 pipeline's 4 launches, the kernel named "
+                                  "and N >= 16384 that is the sort1024 pipeline's 6 launches, the kernel named "
                                   "plus ~20 us of sampler / idle-path launches (profiles/ launch lists)"},
             "issue_roofline": (issue_roofline(kernel_hint, N_rank / (ms_per_step * 1e-3), clk.summary()["sm_mhz"],
                                               torch.cuda.get_device_properties(dev).multi_processor_count)

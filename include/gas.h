@@ -24,8 +24,13 @@
  *     `stream`) from a library-owned memory pool per device that keeps its
  *     memory, so steady-state calls never allocate from the driver and never
  *     synchronise: gas_sort_arrays with 512 < array_len <= 1024 and
- *     num_arrays >= 16384, 4 * num_arrays + 8 bytes; gas_sort_arrays_offsets
- *     with max_array_len > 256, 72 bytes. Everything else: zero workspace.
+ *     num_arrays >= 16384, 4 * num_arrays + 4112 bytes (control block, the
+ *     4 KB batch-CDF table, an array list); with array_len > 16384,
+ *     4 * num_arrays + 8 bytes (n <= 32768) or that plus 64 * num_arrays + 8
+ *     bytes of part offsets and the offsets sort's 72 bytes (n > 32768);
+ *     gas_sort_pairs with 512 < array_len <= 1024, 4 * num_arrays + 4 bytes;
+ *     gas_sort_arrays_offsets with max_array_len > 256, 72 bytes. Everything
+ *     else: zero workspace.
  *   - Work is enqueued on `stream` (0 = legacy default stream) and the call
  *     returns without a host synchronisation. Argument and launch-
  *     configuration errors are returned synchronously; faults during
@@ -77,10 +82,14 @@ typedef enum gas_status {
  *   num_arrays  N >= 0. array_len n >= 0. N == 0 or n <= 1: no-op, d_data may be NULL.
  *   n > gas_max_array_len(): GAS_ERROR_UNSUPPORTED, nothing enqueued.
  * One kernel launch per call, except 512 < n <= 1024 with N >= 16384
- * (BASELINE.json configs[1]-[4]): four launches, a device-routed pipeline
- * (a sampler kernel picks, on the device, which of three kernels sorts the
- * batch: value buckets, counting sort or sorting network; see
- * csrc/sort1024.cuh) and its workspace (above).
+ * (BASELINE.json configs[1]-[4]): a device-routed pipeline of six launches
+ * (four with rows that are not 16-byte aligned): a sampler kernel picks, on
+ * the device, which kernel sorts the batch — value buckets, key-linear
+ * buckets, batch-CDF buckets, the counting sort or the split kernel (special
+ * values and equal-key runs); the others exit at once (csrc/sort1024.cuh);
+ * its workspace is above. 16384 < n <= 65536: two launches (a thread-block
+ * cluster kernel and the fallback for oversize parts), or, for n > 32768, the
+ * partition kernel followed by the variable-length sort's launches.
  */
 GAS_API gas_status gas_sort_arrays(float* d_data, int64_t num_arrays, int32_t array_len, cudaStream_t stream);
 
