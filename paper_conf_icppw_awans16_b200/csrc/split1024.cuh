@@ -44,7 +44,10 @@ namespace gas {
 #ifndef GAS_SP_TMA  // 16-byte rows: stage float bits and leave through one TMA bulk store per array
 #define GAS_SP_TMA 1   // measured: dup16 4.88 -> 4.61 ms, special_mix 6.98 -> 7.11 (only for plain arrays: special_mix 7.69)
 #endif
-constexpr int kSpBlock = 768;                       // 24 warps per SM (as the bucket kernel)
+#ifndef GAS_SP_BLOCK
+#define GAS_SP_BLOCK 640  // measured (profiles/r02_ab_split_block.txt): 512 / 576 / 640 / 704 / 768 threads: dup16 4.56 / 4.69 / 4.50 / 4.82 / 4.61 ms, special_mix 6.82 / 7.71 / 6.95 / 7.73 / 7.13
+#endif
+constexpr int kSpBlock = GAS_SP_BLOCK;              // one block per SM
 constexpr int kSpCntWords = 68;                     // 64 row counters + 4 run counters (-inf, -0, +0, +inf)
 constexpr int kSpCntBytes = kSpCntWords * 4;
 constexpr int kSpRowWords = 36;                     // 32 slots + words 32 / 33: min / max of the overflow keys
