@@ -48,9 +48,7 @@ static __global__ void __launch_bounds__(kBk5Block, 1)
       k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
     }
 #if GAS_BK_PREFETCH
-    if (lane == 0 && a + nwarps < N)
-      asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + (a + nwarps) * (int64_t)n),
-                   "r"((uint32_t)n * 4u) : "memory");
+    bulk_prefetch_elect(a + nwarps < N, d + (a + nwarps) * (int64_t)n, (uint32_t)n * 4u);
 #endif
 #pragma unroll
     for (int q = 2; q < 4; ++q) {
@@ -221,9 +219,10 @@ static __global__ void __launch_bounds__(kBk2Block, 1)
       k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
     }
 #if GAS_BK_PREFETCH
-    if (hl == 0 && a + 2 * nwarps < N)
-      asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(d + (a + 2 * nwarps) * (int64_t)n),
-                   "r"((uint32_t)n * 4u) : "memory");
+    {  // the warp's next pair of arrays, one bulk prefetch by one elected lane
+      const int64_t nb = 2 * (w + nwarps), cnt = N - nb < 2 ? N - nb : 2;
+      bulk_prefetch_elect(nb < N, d + nb * (int64_t)n, (uint32_t)(cnt > 0 ? cnt : 0) * (uint32_t)n * 4u);
+    }
 #endif
 #pragma unroll
     for (int q = 2; q < 4; ++q) {

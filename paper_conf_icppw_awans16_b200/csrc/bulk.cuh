@@ -54,4 +54,30 @@ __device__ __forceinline__ void mbar_wait_parity(uint64_t* bar, uint32_t parity)
   } while (!done);
 }
 
+// One lane (elect.sync: the lowest active lane) issues the bulk operation;
+// no branch, so no BSSY / BSYNC around it (GAS_BK_ELECT). The same lane always
+// wins while the warp is converged, which the bulk-group waits rely on.
+#ifndef GAS_BK_ELECT
+#define GAS_BK_ELECT 1
+#endif
+__device__ __forceinline__ void bulk_prefetch_elect(bool p, const void* g, uint32_t bytes) {
+  asm volatile("{\n\t.reg .pred e, q;\n\telect.sync _|e, 0xffffffff;\n\tsetp.ne.and.u32 q, %2, 0, e;\n\t"
+               "@q cp.async.bulk.prefetch.L2.global [%0], %1;\n\t}"
+               ::"l"(g), "r"(bytes), "r"((uint32_t)p) : "memory");
+}
+__device__ __forceinline__ void bulk_store_elect(void* g, uint32_t sa, uint32_t bytes) {
+  asm volatile("{\n\t.reg .pred e;\n\telect.sync _|e, 0xffffffff;\n\t"
+               "@e cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;\n\t@e cp.async.bulk.commit_group;\n\t}"
+               ::"l"(g), "r"(sa), "r"(bytes) : "memory");
+}
+// prefetch_l2 (the 16-byte-aligned cover of [p, p + words)) issued by one elected lane when `pred`
+__device__ __forceinline__ void prefetch_l2_elect(bool pred, const uint32_t* p, int64_t words) {
+  const uintptr_t a = reinterpret_cast<uintptr_t>(p) & ~(uintptr_t)15;
+  const uintptr_t e = (reinterpret_cast<uintptr_t>(p + words) + 15) & ~(uintptr_t)15;
+  bulk_prefetch_elect(pred, reinterpret_cast<const void*>(a), (uint32_t)(e - a));
+}
+__device__ __forceinline__ void bulk_wait_read_elect() {
+  asm volatile("{\n\t.reg .pred e;\n\telect.sync _|e, 0xffffffff;\n\t@e cp.async.bulk.wait_group.read 0;\n\t}" ::: "memory");
+}
+
 }  // namespace gas

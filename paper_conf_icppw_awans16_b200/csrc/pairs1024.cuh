@@ -83,10 +83,8 @@ __global__ void __launch_bounds__(kPbBlock, 1)
       k[4 * q] = v.x; k[4 * q + 1] = v.y; k[4 * q + 2] = v.z; k[4 * q + 3] = v.w;
     }
 #if GAS_BK_PREFETCH
-    if (lane == 0 && a + nwarps < N) {
-      prefetch_l2(keys + (a + nwarps) * (int64_t)n, n);
-      prefetch_l2(vals + (a + nwarps) * (int64_t)n, n);
-    }
+    prefetch_l2_elect(a + nwarps < N, keys + (a + nwarps) * (int64_t)n, n);
+    prefetch_l2_elect(a + nwarps < N, vals + (a + nwarps) * (int64_t)n, n);
 #endif
 #pragma unroll
     for (int q = 4; q < 8; ++q) {

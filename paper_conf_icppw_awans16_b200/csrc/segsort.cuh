@@ -152,13 +152,10 @@ __global__ void __launch_bounds__(warp_block<G>(), warp_block_min<G>()) k_fixed_
       // no gain for the other classes (profiles/r01_variants_small_prefetch.txt).
       // (unaligned rows: only the 16-byte-aligned interior of the range)
       const int64_t nb = base + nwarps * GROUPS;
-      if (lane == 0 && nb < N) {
-        const int64_t cnt = (N - nb < GROUPS) ? N - nb : GROUPS;
-        const uintptr_t lo = (reinterpret_cast<uintptr_t>(d + nb * (int64_t)n) + 15) & ~uintptr_t(15);
-        const uintptr_t hi = reinterpret_cast<uintptr_t>(d + (nb + cnt) * (int64_t)n) & ~uintptr_t(15);
-        if (hi > lo)
-          asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(lo), "r"((uint32_t)(hi - lo)) : "memory");
-      }
+      const int64_t cnt = (N - nb < GROUPS) ? N - nb : GROUPS;
+      const uintptr_t lo = (reinterpret_cast<uintptr_t>(d + nb * (int64_t)n) + 15) & ~uintptr_t(15);
+      const uintptr_t hi = reinterpret_cast<uintptr_t>(d + (nb + cnt) * (int64_t)n) & ~uintptr_t(15);
+      bulk_prefetch_elect(nb < N && hi > lo, reinterpret_cast<const void*>(lo), (uint32_t)(hi - lo));  // one elected lane
     }
 #endif
     if constexpr (KPT == 32 && G >= 2) sort_group_warp<G>(k, g, reinterpret_cast<uint32_t*>(sb), one);
