@@ -128,6 +128,17 @@ __device__ __forceinline__ void sts32_if(bool p, uint32_t a, uint32_t v) {
   asm volatile("{\n\t.reg .pred q;\n\tsetp.ne.u32 q, %0, 0;\n\t@q st.shared.u32 [%1], %2;\n\t}"
                ::"r"((uint32_t)p), "r"(a), "r"(v) : "memory");
 }
+// Stores the first tb (<= 32) registers of k at consecutive words from word
+// index w0 of the shared array `sw`. The predicates are the bits of a mask, so
+// ptxas sets them 7 at a time with R2P instead of 32 ISETP (GAS_BK_MASKSTORE;
+// plain C++ stores: ordered against the asm shared accesses by their memory
+// clobbers). XF: store bits_from_key of the keys.
+#ifndef GAS_BK_MASKSTORE
+#define GAS_BK_MASKSTORE 1
+#endif
+template <bool XF = false>
+__device__ __forceinline__ void stage_first(uint32_t* sw, uint32_t w0, uint32_t tb, const uint32_t (&k)[32]);
+
 __device__ __forceinline__ uint4 lds128(uint32_t a) {
   uint4 v;
   asm volatile("ld.shared.v4.u32 {%0, %1, %2, %3}, [%4];" : "=r"(v.x), "=r"(v.y), "=r"(v.z), "=r"(v.w) : "r"(a) : "memory");
@@ -135,6 +146,14 @@ __device__ __forceinline__ uint4 lds128(uint32_t a) {
 }
 __device__ __forceinline__ void sts128(uint32_t a, uint4 v) {
   asm volatile("st.shared.v4.u32 [%0], {%1, %2, %3, %4};" ::"r"(a), "r"(v.x), "r"(v.y), "r"(v.z), "r"(v.w) : "memory");
+}
+
+template <bool XF>
+__device__ __forceinline__ void stage_first(uint32_t* sw, uint32_t w0, uint32_t tb, const uint32_t (&k)[32]) {
+  const uint32_t pm = tb >= 32u ? 0xFFFFFFFFu : ((1u << tb) - 1u);
+#pragma unroll
+  for (int i = 0; i < 32; ++i)
+    if (pm & (1u << i)) sw[w0 + i] = XF ? bits_from_key(k[i]) : k[i];
 }
 
 // Bucket map of one value (see the header comment): the bits of
@@ -612,11 +631,21 @@ __global__ void __launch_bounds__(kBkBlock, GAS_BK_WARPS_PER_SM * 32 / kBkBlock)
         for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
         __syncwarp();  // rows 32..63 are drained before any output is staged over them
         sortn_bk<32>(k, one);
+        if (GAS_BK_MASKSTORE && MAP != kMapValue) {  // (the value kernel measured 0.5% slower with it)
+          uint32_t* const sw = reinterpret_cast<uint32_t*>(bk_smem);
+          const uint32_t w0 = (ob - (uint32_t)__cvta_generic_to_shared(bk_smem)) >> 2;
+          if (MAP == kMapKeyLin && GAS_BK_TMA_STORE && !raw) stage_first<true>(sw, w0, tb, k);  // bits (k keeps the keys)
+          else stage_first<false>(sw, w0, tb, k);
+        } else if (MAP == kMapKeyLin && GAS_BK_TMA_STORE && !raw) {  // stage bits (k keeps the keys: they pad the second round)
 #pragma unroll
-        for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
+          for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, bits_from_key(k[i]));
+        } else {
+#pragma unroll
+          for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
+        }
       }
 #if GAS_BK_TMA_STORE
-      if (raw) {  // the staged array is contiguous: one TMA bulk store (the copy engine reads shared memory)
+      if (raw || MAP == kMapKeyLin) {  // the staged array is contiguous: one TMA bulk store (the copy engine reads shared memory)
         asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
         __syncwarp();
         if (GAS_BK_ELECT) {

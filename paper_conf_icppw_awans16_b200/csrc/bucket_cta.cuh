@@ -105,7 +105,10 @@ __device__ __forceinline__ void bar_cta(uint32_t bar) {
 #define GAS_BKC_VOTE_MERGE 1
 #endif
 constexpr uint32_t kBkcOverflow = 0xFFFFFFFFu;  // a warp's scan total when one of its buckets overflowed (totals < 2^31)
-template <int W, int WR, bool VEC, int RV = 16, bool TMA = (GAS_BKC_TMA_STORE != 0)>
+// MASK: staging stores under bitmask predicates (stage_first, bucket1024.cuh):
+// measured faster for one array per CTA (n = 2000 4.60 -> 4.54 ms, configs[3]
+// 5.70 -> 5.68) and slower for the grouped CTAs (n = 4000 4.82 -> 5.08).
+template <int W, int WR, bool VEC, int RV = 16, bool TMA = (GAS_BKC_TMA_STORE != 0), bool MASK = (GAS_BK_MASKSTORE != 0)>
 __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int n, unsigned char* sm, uint32_t one,
                                                 int t, uint32_t bar) {
   using C = BkCta<W, WR>;
@@ -287,7 +290,11 @@ __device__ __forceinline__ void bucket_sort_cta(uint32_t* __restrict__ arr, int 
       // second round reads rows 0 .. T-1, which staging never touches)
       if (rho == 0) bar_cta<WR>(bar);
       sortn_bk<32>(k, one);
-      if (TMA && !raw) {  // the bulk store copies bits: stage transformed keys (k keeps the keys: the
+      if (MASK) {  // bitmask predicates (R2P; stage_first, bucket1024.cuh)
+        uint32_t* const sw = reinterpret_cast<uint32_t*>(sm);
+        if (TMA && !raw) stage_first<true>(sw, (ob - cnt_sa) >> 2, tb, k);
+        else stage_first<false>(sw, (ob - cnt_sa) >> 2, tb, k);
+      } else if (TMA && !raw) {  // the bulk store copies bits: stage transformed keys (k keeps the keys: the
 #pragma unroll            // second round uses them as padding)
         for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, bits_from_key(k[i]));
       } else {
@@ -375,7 +382,8 @@ __global__ void __launch_bounds__(bkc_block<WR>(), bkc_launch_min_blocks<WR>())
 #if GAS_BKC_PREFETCH
     if (t < 32) prefetch_l2_elect(a + stride < N, d + (a + stride) * (int64_t)n, n);
 #endif
-    bucket_sort_cta<W, WR, VEC>(d + a * (int64_t)n, n, sm, one, t, bar);
+    bucket_sort_cta<W, WR, VEC, 16, (GAS_BKC_TMA_STORE != 0), (GAS_BK_MASKSTORE != 0) && !bkc_grouped<WR>()>(
+        d + a * (int64_t)n, n, sm, one, t, bar);
   }
   if (GAS_BKC_TMA_STORE && t == 0) asm volatile("cp.async.bulk.wait_group 0;" ::: "memory");
 }

@@ -191,8 +191,12 @@ __global__ void __launch_bounds__(kS1Block, 1)
         for (int q = 0; q < 8; ++q) lds128_if(4u * q < tb, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
         __syncwarp();  // rows 32..63 are drained before any output is staged over them
         sortn_bk<32>(k, one);
+        if (GAS_BK_MASKSTORE) {
+          stage_first<false>(reinterpret_cast<uint32_t*>(s1_smem), (ob - (uint32_t)__cvta_generic_to_shared(s1_smem)) >> 2, tb, k);
+        } else {
 #pragma unroll
-        for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
+          for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < tb, ob + i * 4, k[i]);
+        }
       }
       __syncwarp();
       if constexpr (!VEC) {

@@ -332,8 +332,13 @@ __global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__
         const bool keys = !over && tb != 0u;
         if (__any_sync(0xffffffffu, keys)) {  // else every row of this round is empty or a run
           if (__any_sync(0xffffffffu, keys && tb >= 2u)) sortn_bk<32>(k, one);
+          if (GAS_BK_MASKSTORE) {
+            uint32_t* const sw = reinterpret_cast<uint32_t*>(sp_smem);
+            stage_first<TB>(sw, (ob - (uint32_t)__cvta_generic_to_shared(sp_smem)) >> 2, keys ? tb : 0u, k);
+          } else {
 #pragma unroll
-          for (int q = 0; q < 32; ++q) sts32_if(keys && (uint32_t)q < tb, ob + q * 4, TB ? bits_from_key(k[q]) : k[q]);
+            for (int q = 0; q < 32; ++q) sts32_if(keys && (uint32_t)q < tb, ob + q * 4, TB ? bits_from_key(k[q]) : k[q]);
+          }
         }
       }
     }
