@@ -393,6 +393,31 @@ def test_cuda_graph_capture_and_replay():
     np.testing.assert_array_equal(to_host(r), expect)
 
 
+@pytest.mark.parametrize("dist", ["paper_uniform", "spectra_intensity", "uniform_bits", "dup16", "special_mix"])
+def test_cuda_graph_pipeline(dist):
+    """The 512 < n <= 1024 pipeline (N >= 16384: sampler, batch-CDF table, path
+    kernels, stream-ordered workspace from the library pool) captured in a CUDA
+    graph and replayed on new data copied into the captured buffer: the sampler
+    re-decides on every replay, every array bit-exact."""
+    N, n = 20000, 1000
+    x = torch.empty((N, n), dtype=torch.float32, device=DEV)
+    s = torch.cuda.Stream()
+    with torch.cuda.stream(s):  # warm-up outside capture (the pool grows here)
+        x.copy_(torch.from_numpy(datagen.fixed(dist, 611, 0, N, n).view(np.float32)))
+        gas.gas_sort_arrays(x)
+    s.synchronize()
+    g = torch.cuda.CUDAGraph()
+    with torch.cuda.graph(g, stream=s):
+        gas.gas_sort_arrays(x)
+    for seed, d in ((612, dist), (613, "paper_uniform"), (614, dist)):  # another distribution in between
+        host = datagen.fixed(d, seed, 0, N, n)
+        x.copy_(torch.from_numpy(host.view(np.float32)))
+        torch.cuda.synchronize()
+        g.replay()
+        torch.cuda.synchronize()
+        np.testing.assert_array_equal(to_host(x.view(torch.int32)).reshape(N, n), oracle_sorted(host))
+
+
 def _offsets_batch(N=3000, seed=77):
     lens = datagen.lengths(seed, 0, N, 100, 4000)
     off = datagen.offsets_from_lengths(lens)
