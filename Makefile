@@ -10,7 +10,7 @@ CSRC := $(wildcard $(PKG)/csrc/*.cu $(PKG)/csrc/*.cuh) include/gas.h
 all: $(PKG)/libgas.so datagen/libgasgen.so oracle/liboracle.so tools/gas_bench
 
 $(PKG)/libgas.so: $(CSRC)
-	$(NVCC) $(NVFLAGS) -shared -Xptxas -warn-spills -I include -o $@ $(PKG)/csrc/gas_api.cu
+	$(NVCC) $(NVFLAGS) -Xcompiler -fvisibility=hidden -shared -Xptxas -warn-spills -I include -o $@ $(wildcard $(PKG)/csrc/*.cu)
 
 datagen/libgasgen.so: datagen/gasgen.cu datagen/gasgen.h
 	$(NVCC) $(ARCH) -O3 -lineinfo -Xcompiler -fPIC -shared -o $@ datagen/gasgen.cu
