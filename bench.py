@@ -443,6 +443,21 @@ def main():
             k = torch.where((b >> 31) == 1, b ^ 0xFFFFFFFF, b ^ 0x80000000)
             ok &= bool((k[:, 1:] >= k[:, :-1]).all())
         del b, k
+    elif ragged:  # flat CSR batch: every adjacent pair inside one array nondecreasing in totalOrder
+        ok = True
+        total = int(off_h[-1] - off_h[0])
+        # first element index of each array -> a pair (j-1, j) crosses an array boundary iff j is an array start
+        starts = torch.zeros(total + 1, dtype=torch.bool, device=dev)
+        starts[(off_d - off_d[0]).clamp(max=total)] = True
+        step = 1 << 28
+        for lo in range(0, total - 1, step):
+            hi = min(total, lo + step + 1)
+            b = work[int(off_h[0]) + lo:int(off_h[0]) + hi].view(torch.int32).to(torch.int64) & 0xFFFFFFFF
+            k = torch.where((b >> 31) == 1, b ^ 0xFFFFFFFF, b ^ 0x80000000)
+            good = (k[1:] >= k[:-1]) | starts[lo + 1:hi]
+            ok &= bool(good.all())
+            del b, k, good
+        del starts
 
     # e2e through the host-buffer C-ABI entry points (pinned memory; copies inside the timed region)
     e2e = None
