@@ -286,11 +286,13 @@ __device__ __forceinline__ uint32_t atoms_add4_if(bool p, uint32_t a) {
 // workspace of one gas_sort_arrays call, followed by an array-index list of
 // up to N entries.
 enum : uint32_t { kS1Bucket = 0, kS1Count = 1, kS1Split = 2, kS1KeyLin = 3, kS1Cdf = 4 };
+enum : uint32_t { kSplitDup = 0, kSplitSpecial = 1 };
 constexpr int kCdfEntries = 512;  // batch CDF table: one entry per (sign, exponent) of the key, i.e. key >> 23
 struct S1Ctl {
   uint32_t flag;      // the path that takes the whole batch (kS1*), written by the sampler
   uint32_t nlist;     // arrays the counting-sort kernel hands to the split kernel (zeroed by the sampler)
-  uint32_t pad[2];
+  uint32_t split_kind;  // kSplitDup / kSplitSpecial: why the sampler chose the split kernel
+  uint32_t pad;
   uint2 cdf[kCdfEntries];  // (A, B) of the batch CDF map (cdf_bucket), written by the sampler
 };
 // The list of nlist array indices follows the control block.

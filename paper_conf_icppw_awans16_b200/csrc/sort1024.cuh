@@ -310,13 +310,13 @@ __device__ __forceinline__ bool bk_sample_dup(uint32_t k0, float vmin, float s) 
 template <bool VEC>
 __global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restrict__ d, int64_t N, int n, S1Ctl* ctl,
                                                            uint32_t force) {
-  __shared__ uint32_t votes[5];  // [0] value fit, [1] key-linear fit, [2] count, [3] split, [4] batch-CDF fit
+  __shared__ uint32_t votes[6];  // [0] value fit, [1] key-linear fit, [2] count, [3] split, [4] batch-CDF fit, [5] special-heavy
   __shared__ uint32_t hist[32][192];  // per warp: value-bucket, key-linear and batch-CDF bucket sizes
   __shared__ uint32_t h512[kCdfEntries];
   __shared__ __align__(8) uint2 tbl[kCdfEntries];
   __shared__ uint32_t part[kCdfEntries / 32];
   const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-  if (threadIdx.x < 5) votes[threadIdx.x] = 0;
+  if (threadIdx.x < 6) votes[threadIdx.x] = 0;
   if (threadIdx.x < kCdfEntries) h512[threadIdx.x] = 0;
   __syncthreads();
   const int64_t S = N < 32 ? N : 32;  // arrays sampled
@@ -373,11 +373,13 @@ __global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restric
       kfit = __reduce_max_sync(0xffffffffu, max(h[64 + lane], h[96 + lane])) <= 32u;
     }
     const uint32_t k0 = bk_sample_key<VEC>(k, lane);
-    const bool to_split = (!raw && s1_sample_special(k0) >= 2) || (ok && bk_sample_dup(k0, vmin, s));
+    const bool special = !raw && s1_sample_special(k0) >= 2;
+    const bool to_split = special || (ok && bk_sample_dup(k0, vmin, s));
     if (lane == 0) {
       if (vfit) atomicAdd(&votes[0], 1u);
       if (kfit) atomicAdd(&votes[1], 1u);
       atomicAdd(&votes[to_split ? 3 : 2], 1u);
+      if (special) atomicAdd(&votes[5], 1u);
     }
   }
   __syncthreads();
@@ -439,6 +441,7 @@ __global__ void __launch_bounds__(1024, 1) k_s1_sample(const uint32_t* __restric
     if (force > kS1Cdf && best == kS1Count) best = votes[3] > votes[2] ? kS1Split : kS1Count;
     ctl->flag = (!VEC && (best == kS1KeyLin || best == kS1Cdf)) ? kS1Count : best;  // those kernels take 16-byte rows only
     ctl->nlist = 0;
+    ctl->split_kind = 2 * votes[5] > votes[3] ? kSplitSpecial : kSplitDup;
   }
 }
 

@@ -164,14 +164,14 @@ __device__ __forceinline__ void sp_fill(uint32_t stage_sa, uint32_t st, uint32_t
 }
 
 // The pipeline's split kernel: the whole batch when ctl->flag == kS1Split,
-// else the arrays the counting-sort kernel listed.
-template <bool VEC>
-__global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one,
-                                                          S1Ctl* ctl) {
-  extern __shared__ __align__(16) uint4 sp_smem[];
-  const uint32_t flag = ctl->flag;
-  const int64_t count = flag == kS1Split ? N : (int64_t)ctl->nlist;
-  if (count == 0) return;
+// else the arrays the counting-sort kernel listed. TB (16-byte rows): stage
+// float bits and leave through one TMA bulk store per array — for batches the
+// sampler found duplicate-heavy (dup16 4.88 -> 4.61 ms); batches it found
+// special-heavy and the listed (special-heavy) arrays keep the key staging
+// (special_mix 6.76 vs 6.95 ms with the bulk store).
+template <bool VEC, bool TB>
+__device__ __forceinline__ void split_body(uint32_t* __restrict__ d, int n, uint32_t one, const S1Ctl* ctl,
+                                           uint32_t flag, int64_t count, uint4* sp_smem) {
   const uint32_t* list = s1_list(ctl);
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const uint32_t wsa = (uint32_t)__cvta_generic_to_shared(sp_smem) + warp * kSpWarpBytes;
@@ -189,7 +189,6 @@ __global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__
     uint32_t* const arr = d + a * (int64_t)n;
     uint32_t k[32];
     s1_load<VEC>(k, arr, n, lane);
-    constexpr bool TB = VEC && GAS_SP_TMA;  // stage bits, bulk store
     if constexpr (TB) {
       bulk_wait_read_elect();  // the previous array's bulk store has read the staging rows
       __syncwarp();
@@ -401,7 +400,20 @@ __global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__
     }
     __syncwarp();
   }
-  if (VEC && GAS_SP_TMA) asm volatile("{\n\t.reg .pred e;\n\telect.sync _|e, 0xffffffff;\n\t@e cp.async.bulk.wait_group 0;\n\t}" ::: "memory");  // bulk stores complete before exit
+  if (TB) asm volatile("{\n\t.reg .pred e;\n\telect.sync _|e, 0xffffffff;\n\t@e cp.async.bulk.wait_group 0;\n\t}" ::: "memory");  // bulk stores complete before exit
+}
+
+template <bool VEC>
+__global__ void __launch_bounds__(kSpBlock, 1) k_s1_split(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one,
+                                                          S1Ctl* ctl) {
+  extern __shared__ __align__(16) uint4 sp_smem[];
+  const uint32_t flag = ctl->flag;
+  const int64_t count = flag == kS1Split ? N : (int64_t)ctl->nlist;
+  if (count == 0) return;
+  if (VEC && GAS_SP_TMA && flag == kS1Split && ctl->split_kind == kSplitDup)
+    split_body<VEC, VEC && GAS_SP_TMA>(d, n, one, ctl, flag, count, sp_smem);
+  else
+    split_body<VEC, false>(d, n, one, ctl, flag, count, sp_smem);
 }
 
 }  // namespace gas
