@@ -45,7 +45,7 @@ namespace gas {
 #define GAS_SP_TMA 1   // measured: dup16 4.88 -> 4.61 ms, special_mix 6.98 -> 7.11 (only for plain arrays: special_mix 7.69)
 #endif
 #ifndef GAS_SP_BLOCK
-#define GAS_SP_BLOCK 640  // measured (profiles/r02_ab_split_block.txt): 512 / 576 / 640 / 704 / 768 threads: dup16 4.56 / 4.69 / 4.50 / 4.82 / 4.61 ms, special_mix 6.82 / 7.71 / 6.95 / 7.73 / 7.13
+#define GAS_SP_BLOCK 512  // measured (profiles/r02_ab_split_block.txt): 384 / 448 / 512 / 640 / 768 threads: dup16 4.94 / 4.81 / 4.53 / 4.57 / 4.85 ms, special_mix 7.83 / 7.59 / 6.61 / 6.74 / 7.14
 #endif
 constexpr int kSpBlock = GAS_SP_BLOCK;              // one block per SM
 constexpr int kSpCntWords = 68;                     // 64 row counters + 4 run counters (-inf, -0, +0, +inf)
