@@ -16,7 +16,7 @@
 namespace gas {
 
 #ifndef GAS_BK5_WARPS
-#define GAS_BK5_WARPS 20  // warps per SM = per block (one block per SM); measured 24: +4%, 16: +3%
+#define GAS_BK5_WARPS 24  // warps per SM = per block (one block per SM); measured (round 2 build): 24 vs 20 vs 16 warps: n = 500 4.197 / 4.213 / 4.260 ms, n = 300 6.072 / 6.124 / 6.198
 #endif
 constexpr int kBk5Block = 32 * GAS_BK5_WARPS;
 constexpr int kBk5CntBytes = 32 * 4;

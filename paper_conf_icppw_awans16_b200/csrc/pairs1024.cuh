@@ -34,7 +34,10 @@
 
 namespace gas {
 
-constexpr int kPbBlock = 384;                         // 12 warps per SM (18.7 KB of shared memory each)
+#ifndef GAS_PB_BLOCK
+#define GAS_PB_BLOCK 384
+#endif
+constexpr int kPbBlock = GAS_PB_BLOCK;                         // 12 warps per SM (18.7 KB of shared memory each)
 constexpr int kPbPosDelta = kBkSlotBytes;             // position rows follow the key rows
 constexpr int kPbWarpBytes = kBkCntBytes + 2 * kBkSlotBytes;
 constexpr int kPbSmemBytes = (kPbBlock / 32) * kPbWarpBytes;
