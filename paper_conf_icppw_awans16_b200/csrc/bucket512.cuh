@@ -134,8 +134,12 @@ static __global__ void __launch_bounds__(kBk5Block, 1)
       __syncwarp();  // every row is drained before the output is staged over them
       sortn_bk<32>(k, one);
       const uint32_t ob = slot_sa + base * 4;
+      if (GAS_BK_MASKSTORE) {
+        stage_first<false>(reinterpret_cast<uint32_t*>(bk5_smem), (ob - (uint32_t)__cvta_generic_to_shared(bk5_smem)) >> 2, t, k);
+      } else {
 #pragma unroll
-      for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < t, ob + i * 4, k[i]);
+        for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < t, ob + i * 4, k[i]);
+      }
       __syncwarp();
       if (raw) {
 #pragma unroll
@@ -297,8 +301,12 @@ static __global__ void __launch_bounds__(kBk2Block, 1)
       __syncwarp();  // every row is drained before the output is staged over them
       sortn_bk<32>(k, one);
       const uint32_t ob = slot_sa + base * 4;
+      if (GAS_BK_MASKSTORE) {
+        stage_first<false>(reinterpret_cast<uint32_t*>(bk2_smem), (ob - (uint32_t)__cvta_generic_to_shared(bk2_smem)) >> 2, t, k);
+      } else {
 #pragma unroll
-      for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < t, ob + i * 4, k[i]);
+        for (int i = 0; i < 32; ++i) sts32_if((uint32_t)i < t, ob + i * 4, k[i]);
+      }
       __syncwarp();
 #pragma unroll
       for (int q = 0; q < 4; ++q) {
