@@ -18,13 +18,21 @@ namespace gas {
 #ifndef GAS_BK5_WARPS
 #define GAS_BK5_WARPS 24  // warps per SM = per block (one block per SM); measured (round 2 build): 24 vs 20 vs 16 warps: n = 500 4.197 / 4.213 / 4.260 ms, n = 300 6.072 / 6.124 / 6.198
 #endif
+#ifndef GAS_BK5_NET16
+// k_fixed_bucket512<NET16 = true> for n <= kBk5Net16MaxN: when every bucket of
+// the warp holds <= 16 keys, the 63-comparator network on k[0..15] instead of
+// 191 (the branch alone costs ~5% where most warps need 32 keys)
+#define GAS_BK5_NET16 1
+#endif
+constexpr int kBk5Net16MaxN = 336;
 constexpr int kBk5Block = 32 * GAS_BK5_WARPS;
 constexpr int kBk5CntBytes = 32 * 4;
 constexpr int kBk5SlotBytes = 32 * kBkRowWords * 4;  // also the fallback network's 4 KB scratch
 constexpr int kBk5WarpBytes = kBk5CntBytes + kBk5SlotBytes;
 constexpr int kBk5SmemBytes = GAS_BK5_WARPS * kBk5WarpBytes;
 
-static __global__ void __launch_bounds__(kBk5Block, 1)
+template <bool NET16>
+__global__ void __launch_bounds__(kBk5Block, 1)
     k_fixed_bucket512(uint32_t* __restrict__ d, int64_t N, int n, uint32_t one) {
   extern __shared__ __align__(16) uint4 bk5_smem[];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -132,7 +140,8 @@ static __global__ void __launch_bounds__(kBk5Block, 1)
 #pragma unroll
       for (int q = 0; q < 8; ++q) lds128_if(4u * q < t, row + q * 16, k[4 * q], k[4 * q + 1], k[4 * q + 2], k[4 * q + 3]);
       __syncwarp();  // every row is drained before the output is staged over them
-      sortn_bk<32>(k, one);
+      if (NET16 && __all_sync(0xffffffffu, t <= 16u)) sortn_bk<16>(k, one);  // rows past 16 keep their pads
+      else sortn_bk<32>(k, one);
       const uint32_t ob = slot_sa + base * 4;
       if (GAS_BK_MASKSTORE) {
         stage_first<false>(reinterpret_cast<uint32_t*>(bk5_smem), (ob - (uint32_t)__cvta_generic_to_shared(bk5_smem)) >> 2, t, k);

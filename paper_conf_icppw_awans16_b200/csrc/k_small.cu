@@ -25,13 +25,21 @@ cudaError_t launch_fixed_warp(uint32_t* d, int64_t N, int n, cudaStream_t s) {
 
 
 // Bucket-then-network kernel for 256 < n <= 512 with aligned rows (bucket512.cuh).
-cudaError_t launch_fixed_bucket512(uint32_t* d, int64_t N, int n, cudaStream_t s) {
-  const cudaError_t attr = set_smem_cached(reinterpret_cast<const void*>(gas::k_fixed_bucket512), gas::kBk5SmemBytes);
+template <bool NET16>
+cudaError_t launch_bucket512(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  auto k = gas::k_fixed_bucket512<NET16>;
+  const cudaError_t attr = set_smem_cached(reinterpret_cast<const void*>(k), gas::kBk5SmemBytes);
   if (attr != cudaSuccess) return attr;
-  const int grid = persistent_grid_smem(gas::k_fixed_bucket512, gas::kBk5Block, gas::kBk5SmemBytes,
-                                        (N + GAS_BK5_WARPS - 1) / GAS_BK5_WARPS);
-  gas::k_fixed_bucket512<<<grid, gas::kBk5Block, gas::kBk5SmemBytes, s>>>(d, N, n, 1u);
+  const int grid = persistent_grid_smem(k, gas::kBk5Block, gas::kBk5SmemBytes, (N + GAS_BK5_WARPS - 1) / GAS_BK5_WARPS);
+  k<<<grid, gas::kBk5Block, gas::kBk5SmemBytes, s>>>(d, N, n, 1u);
   return cudaGetLastError();
+}
+
+// The 16-key network branch only where most warps take it (n = 300: 5.87 ->
+// 5.48 ms; it costs n = 400 / 500 about 5%, profiles/r02_ab_net16.txt).
+cudaError_t launch_fixed_bucket512(uint32_t* d, int64_t N, int n, cudaStream_t s) {
+  if (GAS_BK5_NET16 && n <= gas::kBk5Net16MaxN) return launch_bucket512<true>(d, N, n, s);
+  return launch_bucket512<false>(d, N, n, s);
 }
 
 

@@ -361,3 +361,19 @@ def test_bucket_warp_unaligned(dist, n):
     expect = oracle_sorted(host)
     for lead in (1, 2, 3):
         np.testing.assert_array_equal(gpu_sort_fixed(host, lead=lead), expect)
+
+
+@pytest.mark.parametrize("n,top", [(260, 31), (300, 31), (336, 31), (340, 31), (200, 15)])
+def test_bucket512_256_network_width_edge(n, top):
+    """k_fixed_bucket512<NET16> (n <= 336): the 16-key network (every bucket of
+    the warp <= 16 keys) and the 32-key one (a bucket of 17) on interleaved
+    arrays of one batch, and a bucket of exactly 16 copies of one key; the same
+    rows through the 32-key-only instantiation (n = 340) and bucket256."""
+    rng = np.random.default_rng(500 + n)
+    rows = []
+    for i in range(96):
+        count = (16, 17, 16, 32)[i % 4]
+        hv = np.full(count, 7.0) if i % 8 == 2 else 7.0 + rng.uniform(-0.49, 0.49, size=count)
+        rows.append(spread_array(n, rng, heavy_bucket=7, heavy_count=count, heavy_values=hv, top=top))
+    host = np.stack(rows)
+    np.testing.assert_array_equal(gpu_sort_fixed(host), oracle_sorted(host))
